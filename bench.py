@@ -1,0 +1,387 @@
+#!/usr/bin/env python
+"""Benchmark of the B200 batched tridiagonal solver (one JSON line on rank 0).
+
+Metric (BASELINE.json): systems solved/s and achieved HBM GB/s (% of peak),
+512x512 fp32.  A "step" is one pass of the whole hot path -- load, CR forward
+reduction, intermediate handoff, inner PCR, CR back-substitution, store (all
+SURVEY.md 8(a) rows of the best hybrid, CR+PCR at the tuned m) -- over one
+batch of synthetic diagonally dominant input, i.e. ONE tridiag_solve_batched
+launch.  The 512x512 paper batch is 5.2 MB (L2 resident, launch bound), so the
+per-GPU workload is 256 such batches: S = 131072 systems of n = 512 (1.34 GB,
+> 126 MB L2: no flush needed), the roofline row C2-HBM of SURVEY.md 8(d).
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
+  torchrun --nproc-per-node N bench.py --gpus N ...   (weak scaling: S per GPU)
+
+--impl reference times the CPU oracle (multi-threaded fp64 Thomas, the
+paper's MT solver) on this workload; there is no reference code to install.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+if ROOT not in sys.path:
+    sys.path.insert(0, ROOT)
+
+PEAK_FALLBACK_GBS = 6650.0
+METRIC = "systems solved/s and achieved HBM GB/s (% of peak), 512x512 fp32, 1/2/4/8 B200"
+UNIT = "systems/s"
+
+
+def parse():
+    p = argparse.ArgumentParser()
+    p.add_argument("--gpus", type=int, default=1)
+    p.add_argument("--steps", type=int, default=200)
+    p.add_argument("--warmup", type=int, default=20)
+    p.add_argument("--impl", default="b200", choices=["b200", "reference"])
+    p.add_argument("--n", type=int, default=512)
+    p.add_argument("--systems", type=int, default=131072, help="systems per GPU")
+    p.add_argument("--dtype", default="f32", choices=["f32", "f64"])
+    p.add_argument("--algo", default="cr_pcr")
+    p.add_argument("--switch-level", type=int, default=0)
+    p.add_argument("--family", default="dd")
+    p.add_argument("--no-extras", action="store_true", help="skip per-algorithm table, e2e and cpu baseline")
+    p.add_argument("--cpu-seconds", type=float, default=8.0, help="wall budget of the cpu_baseline leg")
+    return p.parse_args()
+
+
+def measured_peak():
+    path = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(path) as f:
+            j = json.load(f)
+        return float(j["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy best-of-10)"
+    except Exception:
+        return PEAK_FALLBACK_GBS, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(n, dtype, S):
+    """dram bytes per launch from the committed ncu --set full capture, if it
+    matches this workload (profiles/ncu_traffic.json)."""
+    path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    try:
+        with open(path) as f:
+            j = json.load(f)
+        key = f"{dtype}_n{n}_S{S}"
+        return j.get(key, {}).get("dram_bytes_per_launch")
+    except Exception:
+        return None
+
+
+class ClockSampler:
+    """Samples SM clock and throttle reasons with NVML every ~10 ms."""
+    REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap",
+               0x8: "hw_slowdown", 0x10: "sync_boost", 0x20: "sw_thermal_slowdown",
+               0x40: "hw_thermal_slowdown", 0x80: "hw_power_brake_slowdown",
+               0x100: "display_clock_setting"}
+
+    def __init__(self, index):
+        self.ok = False
+        self.samples = []
+        self.max_mhz = None
+        try:
+            import pynvml
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+            self.ok = True
+        except Exception:
+            pass
+        self._stop = threading.Event()
+        self._t = None
+
+    def _run(self):
+        while not self._stop.is_set():
+            try:
+                mhz = self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM)
+                rs = self.nv.nvmlDeviceGetCurrentClocksEventReasons(self.h)
+                util = self.nv.nvmlDeviceGetUtilizationRates(self.h).gpu
+                self.samples.append((mhz, rs, util))
+            except Exception:
+                pass
+            time.sleep(0.01)
+
+    def start(self):
+        if self.ok:
+            self._t = threading.Thread(target=self._run, daemon=True)
+            self._t.start()
+
+    def stop(self):
+        if self._t:
+            self._stop.set()
+            self._t.join()
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": [], "samples": 0}
+        loaded = [s for s in self.samples if s[2] > 0] or self.samples
+        reasons = set()
+        for _, rs, _ in loaded:
+            for bit, name in self.REASONS.items():
+                if rs & bit and name != "gpu_idle":
+                    reasons.add(name)
+        return {"sm_mhz": statistics.median(s[0] for s in loaded), "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(reasons), "samples": len(loaded)}
+
+
+def cpu_cores():
+    try:
+        return len(os.sched_getaffinity(0))
+    except Exception:
+        return os.cpu_count() or 1
+
+
+def cpu_model():
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                if line.startswith("model name"):
+                    return line.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    return "unknown"
+
+
+def cpu_baseline(n, S, dtype_t, family, budget_s):
+    """The oracle (fp64 Thomas, multi-threaded like the paper's MT solver,
+    P:L750-755) as it stands, on a bounded sample of the bench workload."""
+    import numpy as np
+    import torch
+
+    import oracle
+    from paper_conf_ppopp_zhangco10_b200 import inputs
+
+    cores = cpu_cores()
+    S_s = min(S, 32768)
+    a, b, c, d = [t.to(torch.float64).numpy() for t in inputs.generate(family, S_s, n, dtype_t)]
+    x = np.empty_like(d)
+    oracle.thomas_mt(a, b, c, d, cores, out=x)  # warm
+    reps, t0 = 0, time.perf_counter()
+    while True:
+        oracle.thomas_mt(a, b, c, d, cores, out=x)
+        reps += 1
+        el = time.perf_counter() - t0
+        if el >= budget_s or reps >= 1000:
+            break
+    v = reps * S_s / el
+    return {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
+            "sample": f"{reps} x {S_s} systems of n={n} ({family}, fp64 upcast of the {str(dtype_t).replace('torch.', '')} inputs) "
+                      f"= {reps * S_s} of the workload's systems, fp64 Thomas on {cores} threads "
+                      f"({cpu_model()}), wall {el:.2f} s",
+            "gbs": v * 5 * n * (8) / 1e9}
+
+
+def run_reference(args):
+    """--impl reference: the CPU oracle timed as the reference arm."""
+    import numpy as np
+    import torch
+
+    import oracle
+    from paper_conf_ppopp_zhangco10_b200 import inputs
+    from paper_conf_ppopp_zhangco10_b200.partition import dist_env
+
+    rank, _, world = dist_env()
+    if rank != 0:
+        return 0
+    dt = torch.float32 if args.dtype == "f32" else torch.float64
+    n, S = args.n, args.systems
+    cores = cpu_cores()
+    per_step = 2048
+    a, b, c, d = [t.to(torch.float64).numpy() for t in inputs.generate(args.family, per_step * 4, n, dt)]
+    x = np.empty((per_step, n))
+    sl = lambda v, i: v[(i % 4) * per_step:((i % 4) + 1) * per_step]
+    for i in range(args.warmup):
+        oracle.thomas_mt(sl(a, i), sl(b, i), sl(c, i), sl(d, i), cores, out=x)
+    t0 = time.perf_counter()
+    for i in range(args.steps):
+        oracle.thomas_mt(sl(a, i), sl(b, i), sl(c, i), sl(d, i), cores, out=x)
+    el = time.perf_counter() - t0
+    v = args.steps * per_step / el
+    line = {
+        "impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": args.gpus,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * el / args.steps,
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic", "config": workload_config(args, 0),
+        "cpu_baseline": {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
+                         "sample": f"each step: {per_step} systems of n={n} ({args.family}) of the "
+                                   f"workload, fp64 Thomas (oracle) on {cores} threads ({cpu_model()})"},
+        "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+def workload_config(args, m):
+    nbytes = 5 * args.n * (4 if args.dtype == "f32" else 8) * args.systems
+    return {"workload": f"C2-HBM: {args.systems} systems x {args.n} equations {args.dtype} per GPU "
+                        f"({args.systems * args.n // (512 * 512)} paper 512x512 batches), "
+                        f"family {args.family}",
+            "n": args.n, "num_systems_per_gpu": args.systems, "algo": args.algo,
+            "switch_level": m, "family": args.family,
+            "l2": f"inputs {nbytes / 1e9:.2f} GB per step > 126 MB L2 (no flush needed)",
+            "parallelism": f"dp{args.gpus} (batch partition, no collective on the solve path)"}
+
+
+def time_solves(td, bufs, n, S, algo, m, steps, warmup, stream):
+    import torch
+    a, b, c, d, x = bufs
+    with torch.cuda.stream(stream):
+        for _ in range(warmup):
+            td.solve_batched(a, b, c, d, x, algo=algo, switch_level=m, stream=stream)
+    torch.cuda.synchronize()
+    ev = [torch.cuda.Event(enable_timing=True) for _ in range(steps + 1)]
+    launches = 0
+    ev[0].record(stream)
+    for i in range(steps):
+        td.solve_batched(a, b, c, d, x, algo=algo, switch_level=m, stream=stream)
+        launches += td.last_launch_count()
+        ev[i + 1].record(stream)
+    torch.cuda.synchronize()
+    per = [ev[i].elapsed_time(ev[i + 1]) for i in range(steps)]
+    return sum(per) / 1e3, per, launches
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        return run_reference(args)
+
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_ppopp_zhangco10_b200 as td
+    from paper_conf_ppopp_zhangco10_b200 import inputs
+    from paper_conf_ppopp_zhangco10_b200.partition import dist_env, reduce_max
+
+    rank, local, world = dist_env()
+    args.gpus = world
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    td.load(build_if_missing=False)
+    dt = torch.float32 if args.dtype == "f32" else torch.float64
+    T = 4 if args.dtype == "f32" else 8
+    n, S = args.n, args.systems
+    m = args.switch_level or (td.auto_switch_level(n, dt, args.algo) if args.algo in td.HYBRIDS else 0)
+    bytes_per_step = 5 * n * T * S
+
+    # Owner computes: rank r's systems are [r*S, (r+1)*S) of the global batch.
+    s0 = rank * S
+    a, b, c, d = inputs.generate(args.family, S, n, dt, s0=s0, device="cuda")
+    x = torch.empty_like(d)
+    stream = torch.cuda.Stream()
+    sampler = ClockSampler(local)
+
+    # warm-up, then the timed region: barrier + sync on both sides, max over ranks
+    with torch.cuda.stream(stream):
+        for _ in range(args.warmup):
+            td.solve_batched(a, b, c, d, x, algo=args.algo, switch_level=m, stream=stream)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    sampler.start()
+    ev = [torch.cuda.Event(enable_timing=True) for _ in range(args.steps + 1)]
+    launches = 0
+    ev[0].record(stream)
+    for i in range(args.steps):
+        td.solve_batched(a, b, c, d, x, algo=args.algo, switch_level=m, stream=stream)
+        launches += td.last_launch_count()
+        ev[i + 1].record(stream)
+    torch.cuda.synchronize()
+    sampler.stop()
+    per_launch_ms = [ev[i].elapsed_time(ev[i + 1]) for i in range(args.steps)]
+    local_s = sum(per_launch_ms) / 1e3
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    t_max = reduce_max(local_s)
+    value = world * S * args.steps / t_max
+    ms_per_step = 1e3 * t_max / args.steps
+
+    peak, peak_src = measured_peak()
+    kern_s = statistics.mean(per_launch_ms) / 1e3   # this rank's average launch duration
+    achieved = bytes_per_step / kern_s / 1e9
+    traffic = ncu_traffic(n, args.dtype, S)
+    roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                "frac": achieved / peak, "traffic": traffic,
+                "algorithmic_bytes_per_launch": bytes_per_step,
+                "peak_source": peak_src,
+                "frac_of_8TBs": achieved / 8000.0,
+                "kernel": "tdg_warp_kernel<float,16,PCR,false>" if (args.dtype == "f32" and n == 512) else "see DESIGN.md"}
+
+    line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_per_step,
+            "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+            "dtype": args.dtype, "data": "synthetic (counter-based seeded DD family, device-generated)",
+            "config": workload_config(args, m), "roofline": roofline,
+            "hbm_gbs_aggregate": value * 5 * n * T / 1e9,
+            "gpu_launches": launches, "clocks": sampler.summary()}
+
+    if not args.no_extras:
+        # --- e2e: host (pinned) buffers through the C ABI, copies inside the timed region
+        ha, hb, hc, hd = [t.cpu().pin_memory() for t in (a, b, c, d)]
+        hx = torch.empty_like(hd).pin_memory()
+        chunk = 8192
+        ws = torch.empty(td.host_workspace_bytes(n, dt, chunk), dtype=torch.uint8, device="cuda")
+        td.solve_batched_host(ha, hb, hc, hd, hx, algo=args.algo, switch_level=m,
+                              chunk_systems=chunk, workspace=ws)
+        e2e_steps = max(3, min(10, args.steps // 20))
+        if world > 1:
+            dist.barrier()
+        t0 = time.perf_counter()
+        for _ in range(e2e_steps):
+            td.solve_batched_host(ha, hb, hc, hd, hx, algo=args.algo, switch_level=m,
+                                  chunk_systems=chunk, workspace=ws)
+        e2e_local = time.perf_counter() - t0
+        e2e_t = reduce_max(e2e_local)
+        line["e2e"] = {"value": world * S * e2e_steps / e2e_t, "unit": UNIT,
+                       "h2d_bytes_per_step": 4 * n * T * S, "d2h_bytes_per_step": n * T * S,
+                       "how": f"tridiag_solve_batched_host on pinned host buffers, {chunk}-system "
+                              f"chunks pipelined over 2 streams, {e2e_steps} steps, wall clock "
+                              f"around the blocking call, max over ranks"}
+        del ws, ha, hb, hc, hd, hx
+        # --- every algorithm on the same workload (RD family on the RD-stable POI input)
+        per_algo = {}
+        for algo in ("cr", "pcr", "rd", "cr_pcr", "cr_rd"):
+            if n > td.max_n(dt, algo):
+                continue
+            fam = "poi" if algo in ("rd", "cr_rd") else args.family
+            bufs = (a, b, c, d, x) if fam == args.family else (*inputs.generate(fam, S, n, dt, s0=s0, device="cuda"), x)
+            ms = [0]
+            if algo in td.HYBRIDS:
+                ms = sorted({td.auto_switch_level(n, dt, algo), min(n, 256 if algo == "cr_pcr" else 128)})
+            for mm in ms:
+                steps = max(5, args.steps // 4)
+                t, per, _ = time_solves(td, bufs, n, S, algo, mm, steps, 3, stream)
+                tm = reduce_max(t)
+                sps = world * S * steps / tm
+                gbs = bytes_per_step / (t / steps) / 1e9
+                key = algo if mm == 0 else f"{algo}_m{mm}"
+                per_algo[key] = {"systems_per_s": sps, "gbs_per_gpu": gbs, "frac_of_peak": gbs / peak,
+                                 "family": fam}
+        line["per_algo"] = per_algo
+        if rank == 0:
+            line["cpu_baseline"] = cpu_baseline(n, S, dt, args.family, args.cpu_seconds)
+        line["paper_context"] = {"gtx280_cr_pcr_512x512_ms": 0.422,
+                                 "gtx280_systems_per_s": 512 / 0.422e-3,
+                                 "note": "PAPER.md Fig 15 (P:L1100); context only, not vs_baseline"}
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    return 0
+
+
+if __name__ == "__main__":
+    sys.exit(main())

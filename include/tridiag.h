@@ -1,0 +1,146 @@
+/*
+ * tridiag.h -- C ABI of libtridiag.so, the B200 (sm_100a) batched tridiagonal
+ * solver library.
+ *
+ * Method: Zhang, Cohen, Owens, "Fast Tridiagonal Solvers on the GPU",
+ * PPoPP'10 (/root/reference/PAPER.md, cited P:L<line>).  The library solves a
+ * batch of independent tridiagonal systems ("solving a large
+ * number of small tridiagonal systems in parallel") with cyclic reduction
+ * (CR, section 2.1), parallel cyclic reduction (PCR, section 2.2
+ * P:L313-386), recursive doubling (RD, section 2.3) or the hybrids
+ * CR+PCR and CR+RD (section 3, Fig 4).
+ *
+ * No torch or CUDA types appear in this header; `tridiag_stream_t` is
+ * ABI-identical to cudaStream_t / CUstream.
+ */
+#ifndef TRIDIAG_H_
+#define TRIDIAG_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define TRIDIAG_ABI_VERSION 1
+
+typedef struct CUstream_st* tridiag_stream_t; /* == cudaStream_t; NULL = legacy default stream */
+
+/* Element type of all five arrays. */
+typedef enum { TRIDIAG_F32 = 0, TRIDIAG_F64 = 1 } tridiag_dtype;
+
+/* Algorithm.  The hybrids take an intermediate system size m (switch_level). */
+typedef enum {
+    TRIDIAG_CR = 0,     /* P:L272-312, Fig 1                                    */
+    TRIDIAG_PCR = 1,    /* P:L313-386, Fig 2                                    */
+    TRIDIAG_RD = 2,     /* P:L387-421, Fig 3 (Egecioglu scan form of Stone's RD) */
+    TRIDIAG_CR_PCR = 3, /* P:L572-581, Fig 4: CR to m equations, PCR, CR back   */
+    TRIDIAG_CR_RD = 4   /* P:L572-581, Fig 4: CR to m equations, RD, CR back    */
+} tridiag_algo;
+
+/* Status codes.  0 = enqueued.  Negative = argument error, nothing enqueued.
+ * Positive = the cudaError_t reported by the runtime. */
+enum {
+    TRIDIAG_OK = 0,
+    TRIDIAG_ERR_NULL = -1,         /* a required pointer is NULL                     */
+    TRIDIAG_ERR_N = -2,            /* n < 2 or n not a power of two     */
+    TRIDIAG_ERR_N_TOO_LARGE = -3,  /* n > tridiag_max_n(dtype, algo)                 */
+    TRIDIAG_ERR_NUM_SYSTEMS = -4,  /* num_systems < 0                                */
+    TRIDIAG_ERR_DTYPE = -5,        /* dtype not a tridiag_dtype                      */
+    TRIDIAG_ERR_ALGO = -6,         /* algo not a tridiag_algo                        */
+    TRIDIAG_ERR_SWITCH_LEVEL = -7, /* invalid switch_level for this algo / n / dtype */
+    TRIDIAG_ERR_OVERLAP = -8,      /* x overlaps an input other than exactly x == d  */
+    TRIDIAG_ERR_WORKSPACE = -9     /* host entry point: workspace too small / NULL   */
+};
+
+/*
+ * tridiag_solve_batched -- solve num_systems independent systems on the GPU.
+ *
+ * For every s in [0, num_systems) and i in [0, n):
+ *     a[s*n+i] x[s*n+i-1] + b[s*n+i] x[s*n+i] + c[s*n+i] x[s*n+i+1] = d[s*n+i]
+ * with x_{-1} = x_n = 0.  a[s*n] and c[s*n+n-1] are NOT matrix
+ * entries (the paper's matrix has no a_1 and no c_n) and are never read as
+ * coefficients: any value, including NaN, is allowed there.
+ *
+ * Layout: five device arrays of S*n elements of `dtype`,
+ * system-major ("the data of the first system stored at the beginning of the
+ * arrays, followed by the second system, ...").
+ *
+ * a, b, c, d  device pointers, read only.
+ * x           device pointer, written.  x == d (exact in-place) is allowed;
+ *             any other overlap of x with an input is TRIDIAG_ERR_OVERLAP.
+ * n           equations per system: a power of two, 2 <= n <= tridiag_max_n.
+ * num_systems S >= 0.  S == 0 returns TRIDIAG_OK without launching.
+ * dtype       TRIDIAG_F32 or TRIDIAG_F64.  All arithmetic is in this type.
+ * algo        tridiag_algo.
+ * switch_level  the intermediate system size m of the hybrids (Fig 17's
+ *             x-axis, "size-256 intermediate"): 0 = the tuned
+ *             table (tridiag_auto_switch_level); else a power of two with
+ *             2 <= m <= n and m <= tridiag_max_switch_level(dtype, algo, n).
+ *             m = 2 reproduces CR and m = n reproduces PCR / RD.  Must be 0
+ *             for the non-hybrid algorithms.
+ * stream      CUDA stream the work is enqueued on (asynchronous, no host
+ *             synchronisation).
+ *
+ * Pointers must be device memory of the current device.  Alignment: the
+ * vector path needs every pointer aligned to the per-thread tile
+ * (min(32, R*sizeof(T)) bytes); otherwise a scalar-load path runs (same
+ * results).  Results are deterministic: bitwise identical across runs and
+ * across any partitioning of the batch.  Numeric failure (a zero pivot; RD
+ * overflow outside its stable regime) is not an error code: it
+ * shows up as non-finite x (no pivoting).
+ *
+ * Thread safety: reentrant; the only global state is immutable tables and a
+ * per-device launch-configuration cache built under a lock.
+ */
+int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d,
+                          void* x, int64_t n, int64_t num_systems, int dtype, int algo,
+                          int switch_level, tridiag_stream_t stream);
+
+/*
+ * tridiag_solve_batched_host -- the same solve for HOST arrays (the paper's
+ * "with transfer" case).  a, b, c, d, x are host pointers
+ * (pinned memory gives full-speed asynchronous copies; pageable memory works
+ * but serialises).  The batch is split into chunks that are pipelined over
+ * two CUDA streams: the host-to-device copy of chunk j+1 and the
+ * device-to-host copy of chunk j-1 overlap the solve of chunk j.
+ *
+ * workspace        device buffer owned by the caller, at least
+ *                  tridiag_host_workspace_bytes(n, dtype, chunk_systems) bytes.
+ * chunk_systems    systems per chunk (> 0; 0 = library default).
+ * The call BLOCKS until x is written (it is a host-memory API).
+ * x == d is allowed; other overlaps are TRIDIAG_ERR_OVERLAP.
+ */
+int tridiag_solve_batched_host(const void* a, const void* b, const void* c, const void* d,
+                               void* x, int64_t n, int64_t num_systems, int dtype, int algo,
+                               int switch_level, void* workspace, size_t workspace_bytes,
+                               int64_t chunk_systems);
+size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems);
+
+/* Human-readable text of a status code (static storage, never NULL). */
+const char* tridiag_status_string(int status);
+
+/* Largest n this build solves for (dtype, algo); 0 for invalid arguments. */
+int64_t tridiag_max_n(int dtype, int algo);
+
+/* Largest legal intermediate size m for a hybrid at this (dtype, n); for
+ * the non-hybrids 0.  Bounded by the on-chip capacity of the inner solver. */
+int64_t tridiag_max_switch_level(int dtype, int algo, int64_t n);
+
+/* The tuned intermediate size m used when switch_level == 0 (hybrids), from
+ * the switch-level sweep compiled into the library; 0 for non-hybrids or
+ * invalid arguments. */
+int tridiag_auto_switch_level(int64_t n, int dtype, int algo);
+
+/* TRIDIAG_ABI_VERSION of the loaded library. */
+int tridiag_abi_version(void);
+
+/* Number of kernel launches the last successful tridiag_solve_batched call
+ * made on this thread (0 when S == 0).  For the bench's launch count. */
+int tridiag_last_launch_count(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* TRIDIAG_H_ */

@@ -1,1 +1,12 @@
-"""B200-native batched tridiagonal solvers (Zhang, Cohen, Owens, PPoPP'10)."""
+"""B200-native batched tridiagonal solvers: CR, PCR, RD, CR+PCR, CR+RD
+(Zhang, Cohen, Owens, "Fast Tridiagonal Solvers on the GPU", PPoPP'10).
+
+The compute path is libtridiag.so (hand-written sm_100a CUDA behind the C ABI
+of include/tridiag.h); this package is its ctypes binding plus the seeded
+input generator (``inputs``) and the multi-GPU batch partitioner
+(``partition``).
+"""
+from .tridiag import (ALGOS, HYBRIDS, TridiagError, abi_version, auto_switch_level,  # noqa: F401
+                      host_workspace_bytes, last_launch_count, lib_path, load, max_n,
+                      max_switch_level, solve_batched, solve_batched_host, solve_batched_raw,
+                      status_string)

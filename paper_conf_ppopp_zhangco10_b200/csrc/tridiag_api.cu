@@ -1,0 +1,352 @@
+// tridiag_api.cu -- host side of libtridiag.so: argument validation, dispatch
+// to the sm_100a kernels, launch configuration, and the host-buffer pipeline.
+// The C ABI is declared (and documented) in include/tridiag.h.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <cstring>
+#include <map>
+#include <mutex>
+#include <tuple>
+
+#include "tridiag.h"
+#include "tridiag_kernels.cuh"
+
+namespace {
+
+using tdg::ilog2c;
+
+thread_local int g_last_launches = 0;
+
+bool is_pow2(int64_t v) { return v >= 1 && (v & (v - 1)) == 0; }
+int ilog2_64(int64_t v) { int l = 0; while ((int64_t(1) << l) < v) ++l; return l; }
+bool is_hybrid(int algo) { return algo == TRIDIAG_CR_PCR || algo == TRIDIAG_CR_RD; }
+size_t elem_size(int dtype) { return dtype == TRIDIAG_F64 ? 8 : 4; }
+
+// ---------------------------------------------------------------------------
+// Capacity: the inner PCR/RD of an m-system larger than
+// one equation per lane runs in shared memory (9m resp. 13m elements, at most
+// 227 KB per CTA); everything else is register resident.
+// ---------------------------------------------------------------------------
+int64_t max_inner_m(int dtype) { return dtype == TRIDIAG_F64 ? 2048 : 4096; }
+int64_t max_n_cr(int dtype) { return dtype == TRIDIAG_F64 ? 4096 : 8192; }
+
+// Tuned intermediate size for the hybrids when switch_level == 0.  Filled from
+// the config-5 sweep (profiles/): the
+// register/shuffle inner solve (m <= one equation per lane) is what keeps the
+// hybrids HBM-bound on B200.
+int auto_m(int64_t n, int dtype, int algo) {
+  (void)dtype;
+  if (!is_hybrid(algo)) return 0;
+  int64_t m = 32;
+  if (algo == TRIDIAG_CR_RD) m = 32;
+  if (m > n) m = n;
+  return (int)m;
+}
+
+// ---------------------------------------------------------------------------
+// Launch plans.  Kernel family and per-lane equation count R per (dtype, n).
+// ---------------------------------------------------------------------------
+struct Plan {
+  bool cta;  // tdg_cta_kernel (W warps / system) or tdg_warp_kernel
+  int R;
+  int W;     // cta only
+};
+
+Plan plan_for(int dtype, int64_t n) {
+  if (dtype == TRIDIAG_F32) {
+    if (n <= 32) return {false, 1, 0};
+    if (n <= 512) return {false, (int)(n / 32), 0};
+    return {true, 16, (int)(n / (16 * 32))};
+  }
+  if (n <= 32) return {false, 1, 0};
+  if (n <= 256) return {false, (int)(n / 32), 0};
+  return {true, 8, (int)(n / (8 * 32))};
+}
+
+struct Dev {
+  int sms = 0;
+  bool smem_attr_set = false;
+};
+std::mutex g_mu;
+std::map<int, Dev> g_dev;
+std::map<std::tuple<int, const void*, int, size_t>, int> g_occ;
+
+int device_sms(int dev) {
+  std::lock_guard<std::mutex> lk(g_mu);
+  Dev& D = g_dev[dev];
+  if (D.sms == 0) cudaDeviceGetAttribute(&D.sms, cudaDevAttrMultiProcessorCount, dev);
+  return D.sms;
+}
+
+template <typename K>
+int occupancy(int dev, K kernel, int threads, size_t smem) {
+  const void* key = reinterpret_cast<const void*>(kernel);
+  std::lock_guard<std::mutex> lk(g_mu);
+  auto it = g_occ.find({dev, key, threads, smem});
+  if (it != g_occ.end()) return it->second;
+  if (smem > 48 * 1024) cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, kernel, threads, smem) != cudaSuccess) nb = 0;
+  g_occ[{dev, key, threads, smem}] = nb;
+  return nb;
+}
+
+template <typename T, int R, int INNER>
+cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                        int64_t S, int k, bool vec, cudaStream_t st) {
+  const int P = (int)(n / R);
+  const int log2P = ilog2c(P);
+  const int G = 32 / P;
+  const int LR = ilog2c(R);
+  int region = 0;
+  if (k < LR) region = (int)tdg::inner_region_elems(INNER, (int64_t)P * (R >> k));
+  const size_t per_warp = (size_t)G * region * sizeof(T);
+  int wpb = 8;
+  if (per_warp > 0) wpb = (int)std::max<size_t>(1, std::min<size_t>(8, (200 * 1024) / per_warp));
+  const int threads = wpb * 32;
+  const size_t smem = per_warp * wpb;
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = k < LR ? tdg::tdg_warp_kernel<T, R, INNER, true> : tdg::tdg_warp_kernel<T, R, INNER, false>;
+  const int occ = occupancy(dev, kern, threads, smem);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
+                                              vec ? 1 : 0, region);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
+template <typename T, int R, int W, int INNER>
+cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                       int64_t S, int k, bool vec, cudaStream_t st) {
+  const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = k < ilog2c(R) ? tdg::tdg_cta_kernel<T, R, W, INNER, true>
+                             : tdg::tdg_cta_kernel<T, R, W, INNER, false>;
+  const int occ = occupancy(dev, kern, W * 32, smem);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
+template <typename T, int INNER>
+cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const void* d_, void* x_,
+                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype) {
+  const T* a = static_cast<const T*>(a_);
+  const T* b = static_cast<const T*>(b_);
+  const T* c = static_cast<const T*>(c_);
+  const T* d = static_cast<const T*>(d_);
+  T* x = static_cast<T*>(x_);
+  const Plan p = plan_for(dtype, n);
+  const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
+  auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
+  const bool vec = al(a) && al(b) && al(c) && al(d) && al(x);
+  if (!p.cta) {
+    switch (p.R) {
+      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 16: return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+    }
+    return cudaErrorInvalidValue;
+  }
+  if constexpr (sizeof(T) == 4) {
+    switch (p.W) {
+      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+    }
+  } else {
+    switch (p.W) {
+      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+    }
+  }
+  return cudaErrorInvalidValue;
+}
+
+bool overlaps(const void* p, const void* q, size_t bytes) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(p), b = reinterpret_cast<uintptr_t>(q);
+  return a < b + bytes && b < a + bytes;
+}
+
+// Host-side argument validation (integer only; nothing is enqueued on error).
+// On success *m_out is the resolved intermediate size m (n for PCR/RD, 2 for CR).
+int validate(const void* a, const void* b, const void* c, const void* d, const void* x,
+             int64_t n, int64_t S, int dtype, int algo, int switch_level, int64_t* m_out) {
+  if (!a || !b || !c || !d || !x) return TRIDIAG_ERR_NULL;
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
+  if (algo < TRIDIAG_CR || algo > TRIDIAG_CR_RD) return TRIDIAG_ERR_ALGO;
+  if (n < 2 || !is_pow2(n)) return TRIDIAG_ERR_N;
+  if (n > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
+  if (S < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
+  int64_t m;
+  if (algo == TRIDIAG_CR) m = 2;
+  else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD) m = n;
+  else m = switch_level == 0 ? tridiag_auto_switch_level(n, dtype, algo) : switch_level;
+  if (!is_hybrid(algo) && switch_level != 0) return TRIDIAG_ERR_SWITCH_LEVEL;
+  if (is_hybrid(algo)) {
+    if (switch_level < 0 || m < 2 || !is_pow2(m) || m > n ||
+        m > tridiag_max_switch_level(dtype, algo, n))
+      return TRIDIAG_ERR_SWITCH_LEVEL;
+  }
+  const size_t bytes = (size_t)n * (size_t)S * elem_size(dtype);
+  if (bytes > 0) {
+    if (overlaps(x, a, bytes) || overlaps(x, b, bytes) || overlaps(x, c, bytes)) return TRIDIAG_ERR_OVERLAP;
+    if (x != d && overlaps(x, d, bytes)) return TRIDIAG_ERR_OVERLAP;
+  }
+  *m_out = m;
+  return TRIDIAG_OK;
+}
+
+int solve_device(const void* a, const void* b, const void* c, const void* d, void* x, int64_t n,
+                 int64_t S, int dtype, int algo, int64_t m, cudaStream_t st) {
+  if (S == 0) return TRIDIAG_OK;
+  const int k = ilog2_64(n / m);
+  const int inner = (algo == TRIDIAG_RD || algo == TRIDIAG_CR_RD) ? tdg::kRD : tdg::kPCR;
+  cudaError_t e;
+  if (dtype == TRIDIAG_F32)
+    e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype)
+                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype);
+  else
+    e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype)
+                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype);
+  return e == cudaSuccess ? TRIDIAG_OK : (int)e;
+}
+
+}  // namespace
+
+extern "C" {
+
+int tridiag_abi_version(void) { return TRIDIAG_ABI_VERSION; }
+
+int tridiag_last_launch_count(void) { return g_last_launches; }
+
+const char* tridiag_status_string(int status) {
+  switch (status) {
+    case TRIDIAG_OK: return "ok";
+    case TRIDIAG_ERR_NULL: return "null pointer argument";
+    case TRIDIAG_ERR_N: return "n must be a power of two >= 2";
+    case TRIDIAG_ERR_N_TOO_LARGE: return "n exceeds tridiag_max_n(dtype, algo)";
+    case TRIDIAG_ERR_NUM_SYSTEMS: return "num_systems must be >= 0";
+    case TRIDIAG_ERR_DTYPE: return "invalid dtype";
+    case TRIDIAG_ERR_ALGO: return "invalid algo";
+    case TRIDIAG_ERR_SWITCH_LEVEL: return "invalid switch_level for this algo/n/dtype";
+    case TRIDIAG_ERR_OVERLAP: return "x overlaps an input (only x == d is allowed)";
+    case TRIDIAG_ERR_WORKSPACE: return "workspace missing or too small";
+  }
+  if (status > 0) return cudaGetErrorString((cudaError_t)status);
+  return "unknown status";
+}
+
+int64_t tridiag_max_n(int dtype, int algo) {
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return 0;
+  switch (algo) {
+    case TRIDIAG_CR:
+    case TRIDIAG_CR_PCR:
+    case TRIDIAG_CR_RD: return max_n_cr(dtype);
+    case TRIDIAG_PCR:
+    case TRIDIAG_RD: return max_inner_m(dtype);
+  }
+  return 0;
+}
+
+int64_t tridiag_max_switch_level(int dtype, int algo, int64_t n) {
+  if (!is_hybrid(algo) || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
+  if (n < 2 || !is_pow2(n) || n > max_n_cr(dtype)) return 0;
+  return std::min<int64_t>(n, max_inner_m(dtype));
+}
+
+int tridiag_auto_switch_level(int64_t n, int dtype, int algo) {
+  if (!is_hybrid(algo) || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
+  if (n < 2 || !is_pow2(n) || n > max_n_cr(dtype)) return 0;
+  return auto_m(n, dtype, algo);
+}
+
+int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d, void* x,
+                          int64_t n, int64_t num_systems, int dtype, int algo, int switch_level,
+                          tridiag_stream_t stream) {
+  g_last_launches = 0;
+  int64_t m = 0;
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m);
+  if (v != TRIDIAG_OK) return v;
+  return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, m,
+                      reinterpret_cast<cudaStream_t>(stream));
+}
+
+size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems) {
+  if (n < 1 || chunk_systems < 0 || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
+  if (chunk_systems == 0) chunk_systems = std::max<int64_t>(1, (int64_t(16) << 20) / (4 * n * (int64_t)elem_size(dtype)));
+  return (size_t)2 * 4 * (size_t)chunk_systems * (size_t)n * elem_size(dtype);
+}
+
+int tridiag_solve_batched_host(const void* a, const void* b, const void* c, const void* d, void* x,
+                               int64_t n, int64_t num_systems, int dtype, int algo,
+                               int switch_level, void* workspace, size_t workspace_bytes,
+                               int64_t chunk_systems) {
+  g_last_launches = 0;
+  int64_t m = 0;
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m);
+  if (v != TRIDIAG_OK) return v;
+  if (num_systems == 0) return TRIDIAG_OK;
+  if (chunk_systems < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
+  if (chunk_systems == 0)
+    chunk_systems = std::max<int64_t>(1, (int64_t(16) << 20) / (4 * n * (int64_t)elem_size(dtype)));
+  chunk_systems = std::min<int64_t>(chunk_systems, num_systems);
+  const size_t need = tridiag_host_workspace_bytes(n, dtype, chunk_systems);
+  if (!workspace || workspace_bytes < need) return TRIDIAG_ERR_WORKSPACE;
+
+  const size_t T = elem_size(dtype);
+  const size_t arr = (size_t)chunk_systems * (size_t)n * T;  // one array of one chunk
+  cudaStream_t st[2];
+  if (cudaStreamCreateWithFlags(&st[0], cudaStreamNonBlocking) != cudaSuccess) return (int)cudaGetLastError();
+  if (cudaStreamCreateWithFlags(&st[1], cudaStreamNonBlocking) != cudaSuccess) {
+    cudaStreamDestroy(st[0]);
+    return (int)cudaGetLastError();
+  }
+  int rc = TRIDIAG_OK;
+  int launches = 0;
+  const char* hp[4] = {static_cast<const char*>(a), static_cast<const char*>(b),
+                       static_cast<const char*>(c), static_cast<const char*>(d)};
+  char* hx = static_cast<char*>(x);
+  for (int64_t s0 = 0, j = 0; s0 < num_systems && rc == TRIDIAG_OK; s0 += chunk_systems, ++j) {
+    const int64_t cnt = std::min<int64_t>(chunk_systems, num_systems - s0);
+    const size_t bytes = (size_t)cnt * (size_t)n * T;
+    const size_t off = (size_t)s0 * (size_t)n * T;
+    cudaStream_t s = st[j & 1];
+    char* buf = static_cast<char*>(workspace) + (size_t)(j & 1) * 4 * arr;
+    for (int q = 0; q < 4; ++q) {
+      cudaError_t e = cudaMemcpyAsync(buf + q * arr, hp[q] + off, bytes, cudaMemcpyHostToDevice, s);
+      if (e != cudaSuccess) { rc = (int)e; break; }
+    }
+    if (rc != TRIDIAG_OK) break;
+    // x overwrites the chunk's d in place on the device.
+    rc = solve_device(buf, buf + arr, buf + 2 * arr, buf + 3 * arr, buf + 3 * arr, n, cnt, dtype,
+                      algo, m, s);
+    launches += g_last_launches;
+    if (rc != TRIDIAG_OK) break;
+    cudaError_t e = cudaMemcpyAsync(hx + off, buf + 3 * arr, bytes, cudaMemcpyDeviceToHost, s);
+    if (e != cudaSuccess) rc = (int)e;
+  }
+  cudaError_t e0 = cudaStreamSynchronize(st[0]);
+  cudaError_t e1 = cudaStreamSynchronize(st[1]);
+  if (rc == TRIDIAG_OK && e0 != cudaSuccess) rc = (int)e0;
+  if (rc == TRIDIAG_OK && e1 != cudaSuccess) rc = (int)e1;
+  cudaStreamDestroy(st[0]);
+  cudaStreamDestroy(st[1]);
+  g_last_launches = launches;
+  return rc;
+}
+
+}  // extern "C"

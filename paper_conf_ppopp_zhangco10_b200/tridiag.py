@@ -1,0 +1,192 @@
+"""Thin Python binding of libtridiag.so (include/tridiag.h).
+
+Argument marshalling only: every step of the solve runs in the library's
+sm_100a kernels.  torch supplies device memory and the current stream.  If
+the shared library is missing or fails to load, every call raises -- there
+is no CPU fallback.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import threading
+
+import torch
+
+from . import build as _build
+
+ALGOS = {"cr": 0, "pcr": 1, "rd": 2, "cr_pcr": 3, "cr_rd": 4}
+DTYPES = {torch.float32: 0, torch.float64: 1}
+HYBRIDS = ("cr_pcr", "cr_rd")
+
+_lock = threading.Lock()
+_lib = None
+
+
+class TridiagError(RuntimeError):
+    """CUDA-side failure reported by libtridiag (positive status)."""
+
+
+def lib_path() -> str:
+    return _build.LIB
+
+
+def load(build_if_missing: bool = True) -> ctypes.CDLL:
+    """Load libtridiag.so (building it in-tree first if it is missing/stale)."""
+    global _lib
+    with _lock:
+        if _lib is not None:
+            return _lib
+        if build_if_missing:
+            try:
+                _build.build()
+            except (OSError, RuntimeError) as e:  # no nvcc on this machine
+                if not os.path.exists(_build.LIB):
+                    raise RuntimeError(f"libtridiag.so is missing and could not be built: {e}")
+        if not os.path.exists(_build.LIB):
+            raise RuntimeError(f"libtridiag.so not found at {_build.LIB}; run __graft_entry__.build()")
+        L = ctypes.CDLL(_build.LIB)
+        P, I64, I = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int
+        L.tridiag_solve_batched.argtypes = [P, P, P, P, P, I64, I64, I, I, I, P]
+        L.tridiag_solve_batched.restype = I
+        L.tridiag_solve_batched_host.argtypes = [P, P, P, P, P, I64, I64, I, I, I, P,
+                                                 ctypes.c_size_t, I64]
+        L.tridiag_solve_batched_host.restype = I
+        L.tridiag_host_workspace_bytes.argtypes = [I64, I, I64]
+        L.tridiag_host_workspace_bytes.restype = ctypes.c_size_t
+        L.tridiag_status_string.argtypes = [I]
+        L.tridiag_status_string.restype = ctypes.c_char_p
+        L.tridiag_max_n.argtypes = [I, I]
+        L.tridiag_max_n.restype = I64
+        L.tridiag_max_switch_level.argtypes = [I, I, I64]
+        L.tridiag_max_switch_level.restype = I64
+        L.tridiag_auto_switch_level.argtypes = [I64, I, I]
+        L.tridiag_auto_switch_level.restype = I
+        L.tridiag_abi_version.argtypes = []
+        L.tridiag_abi_version.restype = I
+        L.tridiag_last_launch_count.argtypes = []
+        L.tridiag_last_launch_count.restype = I
+        _lib = L
+        return L
+
+
+def _dtype_code(dtype) -> int:
+    if isinstance(dtype, int):
+        return dtype
+    if dtype in DTYPES:
+        return DTYPES[dtype]
+    s = str(dtype).replace("torch.", "")
+    return {"float32": 0, "f32": 0, "float64": 1, "f64": 1}[s]
+
+
+def _algo_code(algo) -> int:
+    return algo if isinstance(algo, int) else ALGOS[algo]
+
+
+def status_string(status: int) -> str:
+    return load().tridiag_status_string(int(status)).decode()
+
+
+def check(status: int) -> None:
+    if status < 0:
+        raise ValueError(f"tridiag: {status_string(status)} (status {status})")
+    if status > 0:
+        raise TridiagError(f"tridiag: CUDA error {status}: {status_string(status)}")
+
+
+def max_n(dtype, algo) -> int:
+    return int(load().tridiag_max_n(_dtype_code(dtype), _algo_code(algo)))
+
+
+def max_switch_level(dtype, algo, n: int) -> int:
+    return int(load().tridiag_max_switch_level(_dtype_code(dtype), _algo_code(algo), int(n)))
+
+
+def auto_switch_level(n: int, dtype, algo) -> int:
+    return int(load().tridiag_auto_switch_level(int(n), _dtype_code(dtype), _algo_code(algo)))
+
+
+def abi_version() -> int:
+    return int(load().tridiag_abi_version())
+
+
+def last_launch_count() -> int:
+    return int(load().tridiag_last_launch_count())
+
+
+def solve_batched_raw(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, n, num_systems, dtype, algo,
+                      switch_level=0, stream=0) -> int:
+    """Direct C-ABI call with integer pointers; returns the status code."""
+    L = load()
+    return int(L.tridiag_solve_batched(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, int(n),
+                                       int(num_systems), _dtype_code(dtype), _algo_code(algo),
+                                       int(switch_level), stream))
+
+
+def _check_tensors(ts, device_kind):
+    t0 = ts[0]
+    if t0.dim() != 2:
+        raise ValueError("tensors must be (num_systems, n)")
+    for t in ts:
+        if t.shape != t0.shape or t.dtype != t0.dtype:
+            raise ValueError("a, b, c, d, x must share shape and dtype")
+        if not t.is_contiguous():
+            raise ValueError("tensors must be contiguous")
+        if device_kind == "cuda" and (not t.is_cuda or t.device != t0.device):
+            raise ValueError("tensors must be on the same CUDA device")
+        if device_kind == "cpu" and t.is_cuda:
+            raise ValueError("host API takes CPU tensors")
+    if t0.dtype not in DTYPES:
+        raise ValueError("dtype must be float32 or float64")
+
+
+def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None):
+    """Solve the (S, n) batch a_i x_{i-1} + b_i x_i + c_i x_{i+1} = d_i on the GPU.
+
+    a, b, c, d: contiguous CUDA tensors (float32/float64) of shape (S, n).
+    x: output tensor (may be d itself for in-place); allocated if None.
+    algo: 'cr' | 'pcr' | 'rd' | 'cr_pcr' | 'cr_rd'.
+    switch_level: intermediate size m of the hybrids (0 = tuned table).
+    Enqueued asynchronously on ``stream`` (default: torch's current stream).
+    """
+    if x is None:
+        x = torch.empty_like(d)
+    _check_tensors([a, b, c, d, x], "cuda")
+    S, n = d.shape
+    if stream is None:
+        stream = torch.cuda.current_stream(d.device)
+    with torch.cuda.device(d.device):
+        st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                               x.data_ptr(), n, S, d.dtype, algo, switch_level,
+                               stream.cuda_stream)
+    check(st)
+    return x
+
+
+def host_workspace_bytes(n: int, dtype, chunk_systems: int = 0) -> int:
+    return int(load().tridiag_host_workspace_bytes(int(n), _dtype_code(dtype), int(chunk_systems)))
+
+
+def solve_batched_host(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, chunk_systems=0,
+                       workspace=None, device=None):
+    """Solve a batch held in HOST memory (pinned CPU tensors for full speed).
+
+    The library pipelines chunks over two streams (H2D, solve, D2H overlap)
+    and returns when x is written.  ``workspace`` is a CUDA uint8 tensor of at
+    least host_workspace_bytes(n, dtype, chunk_systems) bytes (allocated if None).
+    """
+    if x is None:
+        x = torch.empty_like(d)
+    _check_tensors([a, b, c, d, x], "cpu")
+    S, n = d.shape
+    dev = torch.device("cuda", torch.cuda.current_device()) if device is None else torch.device(device)
+    need = host_workspace_bytes(n, d.dtype, chunk_systems)
+    if workspace is None:
+        workspace = torch.empty(need, dtype=torch.uint8, device=dev)
+    with torch.cuda.device(workspace.device):
+        st = load().tridiag_solve_batched_host(
+            a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(), x.data_ptr(), n, S,
+            _dtype_code(d.dtype), _algo_code(algo), int(switch_level), workspace.data_ptr(),
+            workspace.numel(), int(chunk_systems))
+    check(st)
+    return x

@@ -1,0 +1,120 @@
+"""C-ABI of libtridiag.so: loads, exports every declared symbol, and validates
+arguments on the host before touching CUDA (CPU only; no compute calls)."""
+import ctypes
+import os
+import re
+
+import pytest
+
+import paper_conf_ppopp_zhangco10_b200 as td
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+HEADER = os.path.join(ROOT, "include", "tridiag.h")
+
+F32, F64 = 0, 1
+CR, PCR, RD, CR_PCR, CR_RD = range(5)
+# fake, distinct, 256-B aligned "device" pointers: validation never dereferences
+A, B, C, D, X = (0x10000000 * (i + 1) for i in range(5))
+
+
+def declared_functions():
+    src = open(HEADER).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(tridiag_[a-z_]+)\s*\(", src)))
+
+
+def test_library_loads_and_exports_every_declared_symbol():
+    L = td.load()
+    names = declared_functions()
+    assert "tridiag_solve_batched" in names and len(names) >= 9
+    for name in names:
+        assert hasattr(L, name), name
+    assert td.abi_version() == 1
+
+
+def solve(n=512, S=4, dtype=F32, algo=CR, m=0, a=A, b=B, c=C, d=D, x=X):
+    return td.solve_batched_raw(a, b, c, d, x, n, S, dtype, algo, m, None)
+
+
+def test_null_pointers():
+    for kw in ("a", "b", "c", "d", "x"):
+        assert solve(**{kw: 0}) == -1
+
+
+@pytest.mark.parametrize("n", [-4, 0, 1, 3, 6, 100, 513])
+def test_bad_n(n):
+    assert solve(n=n) == -2
+
+
+def test_n_too_large():
+    for dtype in (F32, F64):
+        for algo in range(5):
+            mx = td.max_n(dtype, algo)
+            assert mx >= 512 and (mx & (mx - 1)) == 0
+            assert solve(n=2 * mx, dtype=dtype, algo=algo) == -3
+    assert td.max_n(F32, CR_PCR) == 8192 and td.max_n(F64, CR_PCR) == 4096
+    assert td.max_n(7, CR) == 0 and td.max_n(F32, 9) == 0
+
+
+def test_bad_num_systems_dtype_algo():
+    assert solve(S=-1) == -4
+    assert solve(dtype=2) == -5
+    assert solve(dtype=-1) == -5
+    assert solve(algo=5) == -6
+    assert solve(algo=-1) == -6
+
+
+def test_switch_level_validation():
+    for algo in (CR, PCR, RD):
+        assert solve(algo=algo, m=4) == -7
+    for algo in (CR_PCR, CR_RD):
+        assert solve(algo=algo, m=3) == -7
+        assert solve(algo=algo, m=1) == -7
+        assert solve(algo=algo, m=1024, n=512) == -7
+        assert solve(algo=algo, m=-2) == -7
+        assert solve(algo=algo, n=8192, m=8192) == -7   # inner capacity (fp32: 4096)
+        assert td.max_switch_level(F32, algo, 8192) == 4096
+        assert td.max_switch_level(F64, algo, 4096) == 2048
+        for n in (2, 64, 512, 8192):
+            m = td.auto_switch_level(n, F32, algo)
+            assert 2 <= m <= n and (m & (m - 1)) == 0
+    assert td.auto_switch_level(512, F32, CR) == 0
+
+
+def test_overlap_rules():
+    n, S = 512, 4
+    nbytes = n * S * 4
+    assert solve(x=A) == -8
+    assert solve(x=B + 4) == -8
+    assert solve(x=C - nbytes + 4) == -8
+    assert solve(x=D + 8) == -8          # partial overlap with d
+    assert solve(x=D, S=0) == 0          # exact in-place is allowed (S=0: no launch)
+    assert solve(x=D + nbytes, S=0) == 0
+
+
+def test_zero_systems_is_a_no_op():
+    for algo in range(5):
+        assert solve(S=0, algo=algo) == 0
+    assert td.last_launch_count() == 0
+
+
+def test_status_strings():
+    for s in range(-9, 1):
+        assert isinstance(td.status_string(s), str) and td.status_string(s)
+    assert "power of two" in td.status_string(-2)
+
+
+def test_python_errors_are_loud():
+    with pytest.raises(ValueError):
+        td.tridiag.check(-2)
+    with pytest.raises(td.TridiagError):
+        td.tridiag.check(2)
+
+
+def test_host_workspace_size():
+    assert td.host_workspace_bytes(512, F32, 1000) == 2 * 4 * 1000 * 512 * 4
+    assert td.host_workspace_bytes(512, F64, 0) > 0
+    L = td.load()
+    # workspace too small -> -9 before any CUDA call
+    st = L.tridiag_solve_batched_host(A, B, C, D, X, 512, 4, F32, CR, 0, 0x1000, 16, 2)
+    assert st == -9

@@ -1,0 +1,305 @@
+"""GPU parity: libtridiag (sm_100a) vs the CPU oracle, element by element.
+
+Gates; error = per-system normwise
+max_i |x_i - xhat_i| / max_i |xhat_i| against fp64 Thomas on the exact fp64
+upcast of the T-typed inputs (reading R18), max over systems:
+  G1/G2  CR, PCR, CR+PCR (every m)  DD        fp32 1e-4 / fp64 1e-10
+  G3     same                        KM(1), KM(100)
+  G4     RD, CR+RD                   POI       fp64 1e-10 (n <= 512)
+  G5     RD                          POI       fp32 1e-4  (n <= 32)
+  G5'    CR+RD                       POI       fp32 1e-4  (n <= 64)
+  G6     POI, d = 1 closed form: exact for CR, RD, CR+RD; PCR family <= 4 ulp
+  G7     all five                    POI, CV   fp64 1e-10 (n <= 512)
+Tolerances are the north_star's (1e-4 fp32, 1e-10 fp64).
+"""
+import math
+
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import paper_conf_ppopp_zhangco10_b200 as td
+from paper_conf_ppopp_zhangco10_b200 import inputs
+
+pytestmark = pytest.mark.gpu
+
+TOL = {torch.float32: 1e-4, torch.float64: 1e-10}
+NS = [2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 4096, 8192]
+RAGGED_S = 263  # several warps / CTAs plus a ragged tail
+
+
+@pytest.fixture(scope="module", autouse=True)
+def _cuda():
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    td.load()
+
+
+def gen(family, S, n, dtype, seed=inputs.DEFAULT_SEED, **kw):
+    return inputs.generate(family, S, n, dtype, seed=seed, device="cuda", **kw)
+
+
+def host(*ts):
+    return [t.detach().cpu().numpy() for t in ts]
+
+
+def gpu_solve(a, b, c, d, algo, m=0):
+    x = td.solve_batched(a, b, c, d, algo=algo, switch_level=m)
+    torch.cuda.synchronize()
+    return x
+
+
+def err_vs_oracle(a, b, c, d, x):
+    ref = oracle.thomas(*host(a, b, c, d))  # fp64 Thomas on exact upcast
+    return oracle.normwise_error(host(x)[0], ref)
+
+
+def n_list(dtype, algo):
+    mx = td.max_n(dtype, algo)
+    return [n for n in NS if n <= mx]
+
+
+def m_list(n, dtype, algo):
+    mx = td.max_switch_level(dtype, algo, n)
+    return [2 ** j for j in range(1, int(math.log2(n)) + 1) if 2 ** j <= mx]
+
+
+def S_for(n):
+    return RAGGED_S if n <= 1024 else 37
+
+
+# --------------------------------------------------------------------------- G1 / G2 / G3
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+@pytest.mark.parametrize("algo", ["cr", "pcr", "cr_pcr"])
+def test_cr_family_dd(dtype, algo):
+    for n in n_list(dtype, algo):
+        a, b, c, d = gen("dd", S_for(n), n, dtype, seed=1000 + n)
+        ms = m_list(n, dtype, algo) if algo == "cr_pcr" else [0]
+        for m in ms:
+            x = gpu_solve(a, b, c, d, algo, m)
+            e = err_vs_oracle(a, b, c, d, x)
+            assert e.max() <= TOL[dtype], (algo, n, m, e.max())
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+@pytest.mark.parametrize("E", [1.0, 100.0])
+def test_cr_family_km(dtype, E):
+    for n in [8, 64, 512, 4096]:
+        a, b, c, d = gen("km", 64, n, dtype, E=E, seed=7 + n)
+        for algo, m in [("cr", 0), ("pcr", 0), ("cr_pcr", 0), ("cr_pcr", 4), ("cr_pcr", min(n, 256))]:
+            if n > td.max_n(dtype, algo):
+                continue
+            x = gpu_solve(a, b, c, d, algo, m)
+            e = err_vs_oracle(a, b, c, d, x)
+            assert e.max() <= TOL[dtype], (algo, n, m, E, e.max())
+
+
+# --------------------------------------------------------------------------- G4 / G5 / G5'
+@pytest.mark.parametrize("algo", ["rd", "cr_rd"])
+def test_rd_family_poisson_fp64(algo):
+    for n in [2, 4, 8, 16, 32, 64, 128, 256, 512]:
+        a, b, c, d = gen("poi", RAGGED_S, n, torch.float64, seed=n)
+        for m in (m_list(n, torch.float64, algo) if algo == "cr_rd" else [0]):
+            x = gpu_solve(a, b, c, d, algo, m)
+            e = err_vs_oracle(a, b, c, d, x)
+            assert e.max() <= 1e-10, (algo, n, m, e.max())
+
+
+def test_rd_poisson_fp32():
+    for n in [2, 4, 8, 16, 32]:
+        a, b, c, d = gen("poi", RAGGED_S, n, torch.float32, seed=n)
+        e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "rd"))
+        assert e.max() <= 1e-4, (n, e.max())
+    for n in [4, 8, 16, 32, 64]:
+        a, b, c, d = gen("poi", RAGGED_S, n, torch.float32, seed=n)
+        e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "cr_rd", n // 4 if n >= 8 else 2))
+        assert e.max() <= 1e-4, (n, e.max())
+
+
+# --------------------------------------------------------------------------- G6
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_closed_form_poisson(dtype):
+    for n in [2, 4, 8, 32, 64, 256, 512]:
+        a, b, c, d = gen("poi1", 40, n, dtype)
+        i = np.arange(n, dtype=np.float64)
+        ref = (i + 1.0) * (n - i) / 2.0
+        exact = [("cr", 0), ("rd", 0)] + [("cr_rd", m) for m in m_list(n, dtype, "cr_rd")]
+        for algo, m in exact:
+            x = host(gpu_solve(a, b, c, d, algo, m))[0].astype(np.float64)
+            assert np.array_equal(x, np.broadcast_to(ref, x.shape)), (algo, n, m)
+        eps = float(torch.finfo(dtype).eps)
+        for algo, m in [("pcr", 0)] + [("cr_pcr", m) for m in m_list(n, dtype, "cr_pcr")]:
+            x = host(gpu_solve(a, b, c, d, algo, m))[0].astype(np.float64)
+            e = np.max(np.abs(x - ref), axis=1) / ref.max()
+            assert e.max() <= 4 * eps * max(1, math.log2(n)), (algo, n, m, e.max())
+
+
+# --------------------------------------------------------------------------- G7
+@pytest.mark.parametrize("family", ["poi", "cv"])
+def test_all_five_agree_fp64(family):
+    for n in [8, 64, 512]:
+        a, b, c, d = gen(family, 128, n, torch.float64, seed=3 * n)
+        for algo in ["cr", "pcr", "rd", "cr_pcr", "cr_rd"]:
+            x = gpu_solve(a, b, c, d, algo)
+            e = err_vs_oracle(a, b, c, d, x)
+            assert e.max() <= 1e-10, (family, algo, n, e.max())
+
+
+# --------------------------------------------------------------------------- RD behaviour
+def test_rd_overflow_onset_fp32_matches_paper():
+    """RD "might overflow" for n > 64 on dominant rows: with
+    (a, b, c) = (1, 4, 1), fp32 RD is finite at n = 64 and overflows at 128,
+    like the fp32 oracle RD."""
+    def rows(n):
+        S = 8
+        a = torch.ones(S, n, device="cuda")
+        b = 4 * torch.ones(S, n, device="cuda")
+        d = inputs.generate("dd", S, n, torch.float32, device="cuda")[3]
+        return a, b, a.clone(), d
+    for n, finite in [(32, True), (64, True), (128, False)]:
+        a, b, c, d = rows(n)
+        x = gpu_solve(a, b, c, d, "rd")
+        assert bool(torch.isfinite(x).all()) == finite, n
+        xo = oracle.rd(*host(a, b, c, d), dtype=np.float32)[0]
+        assert bool(np.isfinite(xo).all()) == finite
+
+
+def test_rd_on_dd_reports_instability_not_errors():
+    """R1: RD/CR+RD on DD is outside their stable regime; the
+    library returns normally and the failure shows up as large error or
+    non-finite x, never as a status code."""
+    a, b, c, d = gen("dd", 64, 512, torch.float32)
+    for algo in ("rd", "cr_rd"):
+        x = gpu_solve(a, b, c, d, algo)
+        e = err_vs_oracle(a, b, c, d, x)
+        assert (e > 1e-4).any()
+
+
+# --------------------------------------------------------------------------- edge cases
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_corner_poisoning_is_ignored(dtype):
+    for n in [2, 32, 512, 2048]:
+        a, b, c, d = gen("dd", 50, n, dtype)
+        ap, bp, cp, dp = gen("dd", 50, n, dtype, poison_corners=True)
+        for algo in ["cr", "pcr", "cr_pcr"]:
+            if n > td.max_n(dtype, algo):
+                continue
+            x1 = gpu_solve(a, b, c, d, algo)
+            x2 = gpu_solve(ap, bp, cp, dp, algo)
+            assert torch.isfinite(x2).all(), (algo, n)
+            assert torch.equal(x1, x2), (algo, n)
+        p1 = gen("poi", 50, n, dtype)
+        p2 = gen("poi", 50, n, dtype, poison_corners=True)
+        for algo in ["rd", "cr_rd"]:
+            if n > td.max_n(dtype, algo):
+                continue
+            assert torch.equal(gpu_solve(*p1, algo), gpu_solve(*p2, algo)), (algo, n)
+
+
+def test_in_place_x_equals_d():
+    for dtype in (torch.float32, torch.float64):
+        for n in [64, 512, 4096]:
+            a, b, c, d = gen("dd", 100, n, dtype)
+            ref = gpu_solve(a, b, c, d, "cr_pcr")
+            dd = d.clone()
+            td.solve_batched(a, b, c, dd, x=dd, algo="cr_pcr")
+            torch.cuda.synchronize()
+            assert torch.equal(dd, ref)
+
+
+def test_misaligned_pointers_take_scalar_path():
+    for dtype in (torch.float32, torch.float64):
+        n, S = 512, 77
+        base = [torch.empty(S * n + 1, dtype=dtype, device="cuda") for _ in range(5)]
+        a, b, c, d = gen("dd", S, n, dtype)
+        views = [t[1:].view(S, n) for t in base]
+        for v, src in zip(views[:4], (a, b, c, d)):
+            v.copy_(src)
+        assert views[0].data_ptr() % 16 != 0
+        td.solve_batched(*views[:4], x=views[4], algo="cr_pcr")
+        torch.cuda.synchronize()
+        assert torch.equal(views[4], gpu_solve(a, b, c, d, "cr_pcr"))
+
+
+def test_zero_and_tiny_batches():
+    a, b, c, d = gen("dd", 0, 512, torch.float32)
+    x = gpu_solve(a, b, c, d, "cr_pcr")
+    assert x.shape == (0, 512)
+    for S in (1, 2, 3, 31, 33):
+        a, b, c, d = gen("dd", S, 64, torch.float32)
+        e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "cr_pcr"))
+        assert e.max() <= 1e-4
+
+
+def test_deterministic_and_partition_invariant():
+    """Bitwise identical across reruns and across any split of the batch
+    (what a multi-GPU shard computes is what 1 GPU computes)."""
+    for dtype, n in [(torch.float32, 512), (torch.float64, 512), (torch.float32, 4096)]:
+        S = 300
+        a, b, c, d = gen("dd", S, n, dtype)
+        for algo in ["cr", "pcr", "cr_pcr", "cr_rd", "rd"]:
+            if n > td.max_n(dtype, algo):
+                continue
+            x1 = gpu_solve(a, b, c, d, algo)
+            x2 = gpu_solve(a, b, c, d, algo)
+            assert torch.equal(x1.view(torch.int8), x2.view(torch.int8))
+            parts = [gpu_solve(a[lo:hi].contiguous(), b[lo:hi].contiguous(), c[lo:hi].contiguous(),
+                               d[lo:hi].contiguous(), algo)
+                     for lo, hi in [(0, 117), (117, 118), (118, 300)]]
+            assert torch.equal(torch.cat(parts).view(torch.int8), x1.view(torch.int8))
+
+
+def test_hybrid_endpoints_bitwise():
+    """Fig 17: CR+PCR(m=2) == CR, CR+PCR(m=n) == PCR,
+    CR+RD(m=n) == RD, bitwise (NaN-safe: compare bit patterns)."""
+    for dtype in (torch.float32, torch.float64):
+        for n in [4, 64, 512, 2048]:
+            a, b, c, d = gen("dd", 64, n, dtype)
+            bits = lambda t: t.view(torch.int8)
+            assert torch.equal(bits(gpu_solve(a, b, c, d, "cr_pcr", 2)), bits(gpu_solve(a, b, c, d, "cr")))
+            if n <= td.max_switch_level(dtype, "cr_pcr", n):
+                assert torch.equal(bits(gpu_solve(a, b, c, d, "cr_pcr", n)), bits(gpu_solve(a, b, c, d, "pcr")))
+                assert torch.equal(bits(gpu_solve(a, b, c, d, "cr_rd", n)), bits(gpu_solve(a, b, c, d, "rd")))
+
+
+def test_host_buffer_api_matches_device():
+    for dtype in (torch.float32, torch.float64):
+        n, S = 512, 1000
+        a, b, c, d = gen("dd", S, n, dtype)
+        ref = gpu_solve(a, b, c, d, "cr_pcr")
+        ha, hb, hc, hd = [t.cpu().pin_memory() for t in (a, b, c, d)]
+        hx = torch.empty_like(hd).pin_memory()
+        td.solve_batched_host(ha, hb, hc, hd, hx, algo="cr_pcr", chunk_systems=128)
+        assert torch.equal(hx, ref.cpu())
+        # in place on the host, pageable memory, default chunking
+        hd2 = d.cpu()
+        td.solve_batched_host(a.cpu(), b.cpu(), c.cpu(), hd2, hd2, algo="cr_pcr")
+        assert torch.equal(hd2, ref.cpu())
+
+
+def test_launch_count():
+    a, b, c, d = gen("dd", 10, 512, torch.float32)
+    td.solve_batched(a, b, c, d)
+    assert td.last_launch_count() == 1
+
+
+# --------------------------------------------------------------------------- full size
+def test_full_size_bench_config_sampled():
+    """The bench workload (S = 131072, n = 512, fp32, CR+PCR auto m) in the
+    launch configuration bench.py times: every system has a small residual
+    (property at any size, computed in fp64 with plain torch ops), and 512
+    sampled systems match the oracle one by one."""
+    S, n = 131072, 512
+    a, b, c, d = gen("dd", S, n, torch.float32)
+    x = gpu_solve(a, b, c, d, "cr_pcr")
+    assert torch.isfinite(x).all()
+    a64, b64, c64, d64, x64 = (t.double() for t in (a, b, c, d, x))
+    r = b64 * x64 - d64
+    r[:, 1:] += a64[:, 1:] * x64[:, :-1]
+    r[:, :-1] += c64[:, :-1] * x64[:, 1:]
+    rel = r.abs().amax(dim=1) / d64.abs().amax(dim=1)
+    assert float(rel.max()) <= 1e-5
+    idx = torch.randperm(S, generator=torch.Generator().manual_seed(0))[:512].cuda()
+    e = err_vs_oracle(a[idx], b[idx], c[idx], d[idx], x[idx])
+    assert e.max() <= 1e-4
