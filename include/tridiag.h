@@ -43,7 +43,7 @@ typedef enum {
  * Positive = the cudaError_t reported by the runtime. */
 enum {
     TRIDIAG_OK = 0,
-    TRIDIAG_ERR_NULL = -1,         /* a required pointer is NULL                     */
+    TRIDIAG_ERR_NULL = -1,         /* a pointer is NULL while num_systems > 0        */
     TRIDIAG_ERR_N = -2,            /* n < 2 or n not a power of two     */
     TRIDIAG_ERR_N_TOO_LARGE = -3,  /* n > tridiag_max_n(dtype, algo)                 */
     TRIDIAG_ERR_NUM_SYSTEMS = -4,  /* num_systems < 0                                */
@@ -71,7 +71,8 @@ enum {
  * x           device pointer, written.  x == d (exact in-place) is allowed;
  *             any other overlap of x with an input is TRIDIAG_ERR_OVERLAP.
  * n           equations per system: a power of two, 2 <= n <= tridiag_max_n.
- * num_systems S >= 0.  S == 0 returns TRIDIAG_OK without launching.
+ * num_systems S >= 0.  S == 0 returns TRIDIAG_OK without launching (the
+ *             pointers may then be NULL; the other arguments are validated).
  * dtype       TRIDIAG_F32 or TRIDIAG_F64.  All arithmetic is in this type.
  * algo        tridiag_algo.
  * switch_level  the intermediate system size m of the hybrids (Fig 17's

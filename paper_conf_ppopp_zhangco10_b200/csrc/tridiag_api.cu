@@ -185,7 +185,8 @@ bool overlaps(const void* p, const void* q, size_t bytes) {
 // On success *m_out is the resolved intermediate size m (n for PCR/RD, 2 for CR).
 int validate(const void* a, const void* b, const void* c, const void* d, const void* x,
              int64_t n, int64_t S, int dtype, int algo, int switch_level, int64_t* m_out) {
-  if (!a || !b || !c || !d || !x) return TRIDIAG_ERR_NULL;
+  // NULL pointers are legal only for an empty batch (nothing is accessed).
+  if (S != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
   if (algo < TRIDIAG_CR || algo > TRIDIAG_CR_RD) return TRIDIAG_ERR_ALGO;
   if (n < 2 || !is_pow2(n)) return TRIDIAG_ERR_N;

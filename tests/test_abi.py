@@ -39,6 +39,8 @@ def solve(n=512, S=4, dtype=F32, algo=CR, m=0, a=A, b=B, c=C, d=D, x=X):
 def test_null_pointers():
     for kw in ("a", "b", "c", "d", "x"):
         assert solve(**{kw: 0}) == -1
+        assert solve(S=0, **{kw: 0}) == 0       # empty batch: pointers unused
+    assert solve(S=0, a=0, b=0, c=0, d=0, x=0, n=3) == -2
 
 
 @pytest.mark.parametrize("n", [-4, 0, 1, 3, 6, 100, 513])
