@@ -5,6 +5,7 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <cstring>
 #include <map>
 #include <mutex>
@@ -54,7 +55,20 @@ struct Plan {
   int W;     // cta only
 };
 
+// Tuning knobs (environment, read once): TRIDIAG_WARP_R forces R of the warp
+// kernel when n/R <= 32; TRIDIAG_PREFETCH=0/1 disables/enables the L2 bulk
+// prefetch of the next system.  Defaults come from the sweeps in profiles/.
+int env_int(const char* name, int dflt) {
+  const char* v = getenv(name);
+  return (v && *v) ? atoi(v) : dflt;
+}
+int g_force_R = -1, g_prefetch = -1;
+int force_R() { if (g_force_R < 0) g_force_R = env_int("TRIDIAG_WARP_R", 0); return g_force_R; }
+int prefetch_mode() { if (g_prefetch < 0) g_prefetch = env_int("TRIDIAG_PREFETCH", 2); return g_prefetch; }
+
 Plan plan_for(int dtype, int64_t n) {
+  const int fr = force_R();
+  if (fr > 0 && fr <= 16 && fr <= n && n / fr <= 32 && (fr & (fr - 1)) == 0) return {false, fr, 0};
   if (dtype == TRIDIAG_F32) {
     if (n <= 32) return {false, 1, 0};
     if (n <= 512) return {false, (int)(n / 32), 0};
@@ -114,8 +128,10 @@ cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, in
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
+  const int pm = prefetch_mode();
+  const int pf = vec && (pm == 1 || (pm == 2 && false)) ? 1 : 0;
   kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
-                                              vec ? 1 : 0, region);
+                                              vec ? 1 : 0, region, pf);
   g_last_launches = 1;
   return cudaGetLastError();
 }
@@ -131,7 +147,9 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   const int occ = occupancy(dev, kern, W * 32, smem);
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0);
+  const int pm = prefetch_mode();
+  const int pf = vec && (pm == 1 || pm == 2) ? 1 : 0;
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf);
   g_last_launches = 1;
   return cudaGetLastError();
 }

@@ -73,7 +73,7 @@ template <typename T, int R, int INNER, bool SMEM>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec,
-                int region_elems) {
+                int region_elems, int pf) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   T* smem = reinterpret_cast<T*>(smem_raw);
   const int P = 1 << log2P;
@@ -86,6 +86,13 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
   T* region = smem + (size_t)(warp * G + sub) * region_elems;
   const long long step = (long long)gridDim.x * wpb * G;
   for (long long s0 = ((long long)blockIdx.x * wpb + warp) * G; s0 < S; s0 += step) {
+    if (pf && lane < 4 && s0 + step < S) {
+      // lanes 0..3 prefetch array a, b, c, d of this warp's next group
+      const long long nx = s0 + step;
+      const long long cnt = (S - nx) < G ? (S - nx) : G;
+      const T* base = lane == 0 ? a : lane == 1 ? b : lane == 2 ? c : d;
+      prefetch_l2(base + (size_t)nx * n, (uint32_t)(cnt * n * sizeof(T)));
+    }
     const long long sys = s0 + sub;
     const bool valid = sys < S;
     const size_t off = (size_t)sys * (size_t)n + (size_t)ls * R;
@@ -119,7 +126,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 template <typename T, int R, int W, int INNER, bool SMEM>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-               const T* d, T* x, int n, long long S, int k, int vec) {
+               const T* d, T* x, int n, long long S, int k, int vec, int pf) {
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;
@@ -133,6 +140,12 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
   const int kin = SMEM ? (k < LR ? k : LR) : LR;
 
   for (long long sys = blockIdx.x; sys < S; sys += gridDim.x) {
+    if (pf && lane < 4 && sys + gridDim.x < S) {
+      // lanes 0..3 of every warp prefetch this warp's slice of the next system
+      const T* base = lane == 0 ? a : lane == 1 ? b : lane == 2 ? c : d;
+      prefetch_l2(base + (size_t)(sys + gridDim.x) * n + (size_t)warp * 32 * R,
+                  (uint32_t)(32 * R * sizeof(T)));
+    }
     const size_t off = (size_t)sys * (size_t)n + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
     load_block<T, R, true>(a + off, ra, vec);

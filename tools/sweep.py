@@ -1,0 +1,210 @@
+"""Throughput / accuracy sweeps on one GPU.
+
+  c5     hybrid switch-level sweep: S = 16384, n = 128..8192, fp32/fp64,
+         CR+PCR and CR+RD at every valid m; throughput on DD (CR+RD on POI)
+         plus max normwise error vs the oracle on DD and POI samples.
+  c2     all five algorithms at n = 64..512 on HBM-scale batches (S*n = 2^26)
+         and the literal paper shapes S = n (L2-resident; CUDA graph of 100
+         launches over rotating buffer sets -> us per batch).
+  c3     ADI-style 4096 x 4096, fp32 and fp64, all algorithms that fit.
+  c4     2^20 x 256 fp32 on one GPU (the W = 1 point of the scaling row).
+
+Writes one JSON object per point to stdout.  Timing: CUDA events on the
+launching stream, warm-up first, working set >= 4x L2 via rotating buffer sets.
+"""
+import argparse
+import json
+import math
+import os
+import statistics
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+import numpy as np  # noqa: E402
+import torch  # noqa: E402
+
+import oracle  # noqa: E402
+import paper_conf_ppopp_zhangco10_b200 as td  # noqa: E402
+from paper_conf_ppopp_zhangco10_b200 import inputs  # noqa: E402
+
+L2_BYTES = 126 * 1024 * 1024
+PEAK = 6547.5
+try:
+    PEAK = float(json.load(open(os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))),
+                                             "MEASURED_PEAKS.json")))["hbm_gbs"])
+except Exception:
+    pass
+
+
+def make_sets(family, S, n, dt, min_bytes):
+    T = 4 if dt == torch.float32 else 8
+    per = 5 * S * n * T
+    nsets = max(1, math.ceil(min_bytes / per))
+    nsets = min(nsets, 64)
+    sets = []
+    for k in range(nsets):
+        a, b, c, d = inputs.generate(family, S, n, dt, s0=k * S, device="cuda")
+        sets.append((a, b, c, d, torch.empty_like(d)))
+    return sets, per
+
+
+def time_point(sets, algo, m, steps=50, warmup=5):
+    st = torch.cuda.current_stream()
+    for i in range(warmup):
+        a, b, c, d, x = sets[i % len(sets)]
+        td.solve_batched(a, b, c, d, x, algo=algo, switch_level=m)
+    torch.cuda.synchronize()
+    ev = [torch.cuda.Event(enable_timing=True) for _ in range(steps + 1)]
+    ev[0].record(st)
+    for i in range(steps):
+        a, b, c, d, x = sets[i % len(sets)]
+        td.solve_batched(a, b, c, d, x, algo=algo, switch_level=m)
+        ev[i + 1].record(st)
+    torch.cuda.synchronize()
+    per = [ev[i].elapsed_time(ev[i + 1]) * 1e-3 for i in range(steps)]
+    return statistics.median(per), min(per)
+
+
+def accuracy(family, n, dt, algo, m, S=256, **kw):
+    a, b, c, d = inputs.generate(family, S, n, dt, device="cuda", seed=4242, **kw)
+    x = td.solve_batched(a, b, c, d, algo=algo, switch_level=m)
+    torch.cuda.synchronize()
+    ha, hb, hc, hd = [t.cpu().numpy() for t in (a, b, c, d)]
+    ref = oracle.thomas(ha, hb, hc, hd)
+    e = oracle.normwise_error(x.cpu().numpy(), ref)
+    fin = np.isfinite(e)
+    res = oracle.residual_inf(ha, hb, hc, hd, x.cpu().numpy().astype(np.float64))
+    return {"max_err": float(e[fin].max()) if fin.any() else None,
+            "nonfinite": int((~fin).sum()), "systems": S,
+            "max_residual": float(np.nanmax(res)) if fin.any() else None}
+
+
+def emit(d):
+    print(json.dumps(d), flush=True)
+
+
+def c5(args):
+    S = 16384
+    for dts in ("f32", "f64"):
+        dt = torch.float32 if dts == "f32" else torch.float64
+        for n in [128, 256, 512, 1024, 2048, 4096, 8192]:
+            for algo in ("cr_pcr", "cr_rd"):
+                if n > td.max_n(dt, algo):
+                    continue
+                fam = "dd" if algo == "cr_pcr" else "poi"
+                sets, per = make_sets(fam, S, n, dt, 4 * L2_BYTES)
+                mx = td.max_switch_level(dt, algo, n)
+                for lm in range(1, int(math.log2(n)) + 1):
+                    m = 2 ** lm
+                    if m > mx:
+                        continue
+                    med, mn = time_point(sets, algo, m, steps=args.steps)
+                    row = {"config": "c5", "dtype": dts, "n": n, "S": S, "algo": algo, "m": m,
+                           "time_family": fam, "ms_median": med * 1e3, "ms_min": mn * 1e3,
+                           "systems_per_s": S / med, "gbs": per / med / 1e9,
+                           "frac_of_peak": per / med / 1e9 / PEAK,
+                           "auto": m == td.auto_switch_level(n, dt, algo)}
+                    if not args.no_acc:
+                        row["acc_dd"] = accuracy("dd", n, dt, algo, m)
+                        row["acc_poi"] = accuracy("poi", n, dt, algo, m)
+                    emit(row)
+                del sets
+                torch.cuda.empty_cache()
+
+
+def c2(args):
+    dt = torch.float32
+    for n in [64, 128, 256, 512]:
+        S = (1 << 26) // n
+        for algo in ("cr", "pcr", "rd", "cr_pcr", "cr_rd"):
+            fam = "poi" if algo in ("rd", "cr_rd") else "dd"
+            sets, per = make_sets(fam, S, n, dt, 0)
+            ms = [0]
+            if algo in td.HYBRIDS:
+                ms = sorted({td.auto_switch_level(n, dt, algo), n // 2, 256 if algo == "cr_pcr" else 128} & set(
+                    2 ** j for j in range(1, int(math.log2(n)) + 1)))
+            for m in ms:
+                med, mn = time_point(sets, algo, m, steps=args.steps)
+                emit({"config": "c2-hbm", "dtype": "f32", "n": n, "S": S, "algo": algo, "m": m,
+                      "time_family": fam, "ms_median": med * 1e3, "systems_per_s": S / med,
+                      "gbs": per / med / 1e9, "frac_of_peak": per / med / 1e9 / PEAK})
+            del sets
+        torch.cuda.empty_cache()
+    # literal paper shapes: S = n, L2 resident; graph of 100 launches on rotating sets
+    for n in [64, 128, 256, 512]:
+        S = n
+        for algo in ("cr", "pcr", "rd", "cr_pcr", "cr_rd"):
+            fam = "poi" if algo in ("rd", "cr_rd") else "dd"
+            sets, per = make_sets(fam, S, n, dt, 4 * L2_BYTES)
+            g = torch.cuda.CUDAGraph()
+            st = torch.cuda.Stream()
+            with torch.cuda.stream(st):
+                for i in range(3):
+                    a, b, c, d, x = sets[i % len(sets)]
+                    td.solve_batched(a, b, c, d, x, algo=algo)
+            torch.cuda.synchronize()
+            with torch.cuda.graph(g, stream=st):
+                for i in range(100):
+                    a, b, c, d, x = sets[i % len(sets)]
+                    td.solve_batched(a, b, c, d, x, algo=algo, stream=st)
+            g.replay()
+            torch.cuda.synchronize()
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record()
+            for _ in range(5):
+                g.replay()
+            e1.record()
+            torch.cuda.synchronize()
+            us = e0.elapsed_time(e1) * 1e3 / 500
+            emit({"config": "c2-literal", "dtype": "f32", "n": n, "S": S, "algo": algo,
+                  "m": td.auto_switch_level(n, dt, algo) if algo in td.HYBRIDS else 0,
+                  "us_per_batch": us, "systems_per_s": S / (us * 1e-6),
+                  "paper_gtx280_ms": {"cr": 1.066, "pcr": 0.534, "rd": 0.612, "cr_pcr": 0.422,
+                                      "cr_rd": 0.488}[algo] if n == 512 else None})
+            del sets, g
+        torch.cuda.empty_cache()
+
+
+def c3(args):
+    n, S = 4096, 4096
+    for dts in ("f32", "f64"):
+        dt = torch.float32 if dts == "f32" else torch.float64
+        for algo in ("cr", "pcr", "rd", "cr_pcr", "cr_rd"):
+            if n > td.max_n(dt, algo):
+                continue
+            fam = "poi" if algo in ("rd", "cr_rd") else "dd"
+            sets, per = make_sets(fam, S, n, dt, 4 * L2_BYTES)
+            med, mn = time_point(sets, algo, 0, steps=args.steps)
+            row = {"config": "c3", "dtype": dts, "n": n, "S": S, "algo": algo,
+                   "m": td.auto_switch_level(n, dt, algo) if algo in td.HYBRIDS else 0,
+                   "time_family": fam, "ms_median": med * 1e3, "systems_per_s": S / med,
+                   "gbs": per / med / 1e9, "frac_of_peak": per / med / 1e9 / PEAK}
+            if not args.no_acc:
+                row["acc"] = accuracy(fam, n, dt, algo, 0, S=64)
+            emit(row)
+            del sets
+            torch.cuda.empty_cache()
+
+
+def c4(args):
+    n, S = 256, 1 << 20
+    dt = torch.float32
+    sets, per = make_sets("dd", S, n, dt, 0)
+    for algo in ("cr", "cr_pcr"):
+        med, mn = time_point(sets, algo, 0, steps=args.steps)
+        emit({"config": "c4-w1", "dtype": "f32", "n": n, "S": S, "algo": algo,
+              "m": td.auto_switch_level(n, dt, algo) if algo in td.HYBRIDS else 0,
+              "ms_median": med * 1e3, "systems_per_s": S / med, "gbs": per / med / 1e9,
+              "frac_of_peak": per / med / 1e9 / PEAK})
+
+
+if __name__ == "__main__":
+    p = argparse.ArgumentParser()
+    p.add_argument("configs", nargs="+", choices=["c2", "c3", "c4", "c5"])
+    p.add_argument("--steps", type=int, default=30)
+    p.add_argument("--no-acc", action="store_true")
+    a = p.parse_args()
+    td.load(build_if_missing=False)
+    for cfg in a.configs:
+        globals()[cfg](a)
