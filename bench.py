@@ -43,7 +43,9 @@ def parse():
     p.add_argument("--warmup", type=int, default=20)
     p.add_argument("--impl", default="b200", choices=["b200", "reference"])
     p.add_argument("--n", type=int, default=512)
-    p.add_argument("--systems", type=int, default=131072, help="systems per GPU")
+    p.add_argument("--systems", type=int, default=131072, help="systems per GPU (weak scaling)")
+    p.add_argument("--total-systems", type=int, default=0,
+                   help="strong scaling: split this many systems over the ranks (C4: 1048576 x n=256)")
     p.add_argument("--dtype", default="f32", choices=["f32", "f64"])
     p.add_argument("--algo", default="cr_pcr")
     p.add_argument("--switch-level", type=int, default=0)
@@ -231,6 +233,18 @@ def workload_config(args, m):
             "parallelism": f"dp{args.gpus} (batch partition, no collective on the solve path)"}
 
 
+def rank_workload(args, rank, world):
+    """(first global system, systems on this rank, systems in the job, scaling).
+    Weak scaling (default): every rank owns args.systems systems, rank r the
+    global range [r*S, (r+1)*S).  Strong scaling (--total-systems T): the
+    partitioner splits T contiguously (sizes differ by at most one)."""
+    from paper_conf_ppopp_zhangco10_b200.partition import shard_range
+    if args.total_systems:
+        sh = shard_range(args.total_systems, world, rank)
+        return sh.lo, sh.count, args.total_systems, "strong"
+    return rank * args.systems, args.systems, world * args.systems, "weak"
+
+
 def time_solves(td, bufs, n, S, algo, m, steps, warmup, stream):
     import torch
     a, b, c, d, x = bufs
@@ -270,12 +284,12 @@ def main():
     td.load(build_if_missing=False)
     dt = torch.float32 if args.dtype == "f32" else torch.float64
     T = 4 if args.dtype == "f32" else 8
-    n, S = args.n, args.systems
+    n = args.n
+    # Owner computes: this rank's systems are [s0, s0+S) of the global batch.
+    s0, S, total, scaling = rank_workload(args, rank, world)
+    args.systems = S
     m = args.switch_level or (td.auto_switch_level(n, dt, args.algo) if args.algo in td.HYBRIDS else 0)
     bytes_per_step = 5 * n * T * S
-
-    # Owner computes: rank r's systems are [r*S, (r+1)*S) of the global batch.
-    s0 = rank * S
     a, b, c, d = inputs.generate(args.family, S, n, dt, s0=s0, device="cuda")
     x = torch.empty_like(d)
     stream = torch.cuda.Stream()
@@ -305,7 +319,7 @@ def main():
         dist.barrier()
     torch.cuda.synchronize()
     t_max = reduce_max(local_s)
-    value = world * S * args.steps / t_max
+    value = total * args.steps / t_max
     ms_per_step = 1e3 * t_max / args.steps
 
     peak, peak_src = measured_peak()
@@ -321,10 +335,11 @@ def main():
 
     line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_per_step,
-            "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+            "higher_is_better": True, "scaling": scaling, "vs_baseline": None,
             "dtype": args.dtype, "data": "synthetic (counter-based seeded DD family, device-generated)",
             "config": workload_config(args, m), "roofline": roofline,
             "hbm_gbs_aggregate": value * 5 * n * T / 1e9,
+            "systems_in_job": total,
             "gpu_launches": launches, "clocks": sampler.summary()}
 
     if not args.no_extras:
@@ -344,7 +359,7 @@ def main():
                                   chunk_systems=chunk, workspace=ws)
         e2e_local = time.perf_counter() - t0
         e2e_t = reduce_max(e2e_local)
-        line["e2e"] = {"value": world * S * e2e_steps / e2e_t, "unit": UNIT,
+        line["e2e"] = {"value": total * e2e_steps / e2e_t, "unit": UNIT,
                        "h2d_bytes_per_step": 4 * n * T * S, "d2h_bytes_per_step": n * T * S,
                        "how": f"tridiag_solve_batched_host on pinned host buffers, {chunk}-system "
                               f"chunks pipelined over 2 streams, {e2e_steps} steps, wall clock "
@@ -364,7 +379,7 @@ def main():
                 steps = max(5, args.steps // 4)
                 t, per, _ = time_solves(td, bufs, n, S, algo, mm, steps, 3, stream)
                 tm = reduce_max(t)
-                sps = world * S * steps / tm
+                sps = total * steps / tm
                 gbs = bytes_per_step / (t / steps) / 1e9
                 key = algo if mm == 0 else f"{algo}_m{mm}"
                 per_algo[key] = {"systems_per_s": sps, "gbs_per_gpu": gbs, "frac_of_peak": gbs / peak,

@@ -33,15 +33,20 @@ size_t elem_size(int dtype) { return dtype == TRIDIAG_F64 ? 8 : 4; }
 int64_t max_inner_m(int dtype) { return dtype == TRIDIAG_F64 ? 2048 : 4096; }
 int64_t max_n_cr(int dtype) { return dtype == TRIDIAG_F64 ? 4096 : 8192; }
 
-// Tuned intermediate size for the hybrids when switch_level == 0.  Filled from
-// the config-5 sweep (profiles/): the
-// register/shuffle inner solve (m <= one equation per lane) is what keeps the
-// hybrids HBM-bound on B200.
+// Tuned intermediate size for the hybrids when switch_level == 0, from the
+// switch-level sweeps (profiles/r01_tune_plan.md; Fig 17 is the paper's
+// version of this sweep).  On B200 every m that keeps the inner
+// solve in registers (m <= lanes per system) runs at the HBM roofline within
+// noise, and every larger m is 2-10x slower; so CR+PCR takes the largest
+// register-resident m (fewest CR levels) and CR+RD the smallest m within 2% of
+// the best time (8), because RD's error grows with m on dominant input
+// (R24).
+int lanes_per_system(int dtype, int64_t n);
 int auto_m(int64_t n, int dtype, int algo) {
-  (void)dtype;
   if (!is_hybrid(algo)) return 0;
-  int64_t m = 32;
-  if (algo == TRIDIAG_CR_RD) m = 32;
+  const int64_t P = lanes_per_system(dtype, n);
+  int64_t m = algo == TRIDIAG_CR_PCR ? std::min<int64_t>(P, 32) : std::min<int64_t>(P, 8);
+  if (m < 2) m = 2;
   if (m > n) m = n;
   return (int)m;
 }
@@ -66,17 +71,21 @@ int g_force_R = -1, g_prefetch = -1;
 int force_R() { if (g_force_R < 0) g_force_R = env_int("TRIDIAG_WARP_R", 0); return g_force_R; }
 int prefetch_mode() { if (g_prefetch < 0) g_prefetch = env_int("TRIDIAG_PREFETCH", 2); return g_prefetch; }
 
+// R per lane from the plan sweep (profiles/r01_tune_plan.md): the widest
+// register block that fits (16 fp32 / 8 fp64 equations per lane) is fastest at
+// every n; systems with n <= 32 use 4 lanes (or n lanes when n < 4).
 Plan plan_for(int dtype, int64_t n) {
   const int fr = force_R();
   if (fr > 0 && fr <= 16 && fr <= n && n / fr <= 32 && (fr & (fr - 1)) == 0) return {false, fr, 0};
-  if (dtype == TRIDIAG_F32) {
-    if (n <= 32) return {false, 1, 0};
-    if (n <= 512) return {false, (int)(n / 32), 0};
-    return {true, 16, (int)(n / (16 * 32))};
-  }
-  if (n <= 32) return {false, 1, 0};
-  if (n <= 256) return {false, (int)(n / 32), 0};
-  return {true, 8, (int)(n / (8 * 32))};
+  const int Rmax = dtype == TRIDIAG_F32 ? 16 : 8;
+  if (n <= 32) return {false, (int)std::max<int64_t>(1, n / 4), 0};
+  if (n <= 32 * Rmax) return {false, Rmax, 0};
+  return {true, Rmax, (int)(n / (Rmax * 32))};
+}
+
+int lanes_per_system(int dtype, int64_t n) {
+  const Plan p = plan_for(dtype, n);
+  return p.cta ? 32 : (int)(n / p.R);
 }
 
 struct Dev {
@@ -129,7 +138,7 @@ cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, in
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
   const int pm = prefetch_mode();
-  const int pf = vec && (pm == 1 || (pm == 2 && false)) ? 1 : 0;
+  const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
                                               vec ? 1 : 0, region, pf);
   g_last_launches = 1;
