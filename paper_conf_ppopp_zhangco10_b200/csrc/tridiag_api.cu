@@ -76,8 +76,8 @@ int prefetch_mode() { if (g_prefetch < 0) g_prefetch = env_int("TRIDIAG_PREFETCH
 // every n; systems with n <= 32 use 4 lanes (or n lanes when n < 4).
 Plan plan_for(int dtype, int64_t n) {
   const int fr = force_R();
-  if (fr > 0 && fr <= 16 && fr <= n && n / fr <= 32 && (fr & (fr - 1)) == 0) return {false, fr, 0};
   const int Rmax = dtype == TRIDIAG_F32 ? 16 : 8;
+  if (fr > 0 && fr <= Rmax && fr <= n && n / fr <= 32 && (fr & (fr - 1)) == 0) return {false, fr, 0};
   if (n <= 32) return {false, (int)std::max<int64_t>(1, n / 4), 0};
   if (n <= 32 * Rmax) return {false, Rmax, 0};
   return {true, Rmax, (int)(n / (Rmax * 32))};
@@ -116,33 +116,43 @@ int occupancy(int dev, K kernel, int threads, size_t smem) {
   return nb;
 }
 
-template <typename T, int R, int INNER>
-cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                        int64_t S, int k, bool vec, cudaStream_t st) {
+template <typename T, int R, int INNER, int KB>
+cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                          int64_t S, int k, bool vec, cudaStream_t st) {
   const int P = (int)(n / R);
   const int log2P = ilog2c(P);
   const int G = 32 / P;
-  const int LR = ilog2c(R);
-  int region = 0;
-  if (k < LR) region = (int)tdg::inner_region_elems(INNER, (int64_t)P * (R >> k));
-  const size_t per_warp = (size_t)G * region * sizeof(T);
-  int wpb = 8;
-  if (per_warp > 0) wpb = (int)std::max<size_t>(1, std::min<size_t>(8, (200 * 1024) / per_warp));
+  const int wpb = 8;
   const int threads = wpb * 32;
-  const size_t smem = per_warp * wpb;
   int dev = 0;
   cudaGetDevice(&dev);
-  auto kern = k < LR ? tdg::tdg_warp_kernel<T, R, INNER, true> : tdg::tdg_warp_kernel<T, R, INNER, false>;
-  const int occ = occupancy(dev, kern, threads, smem);
+  auto kern = tdg::tdg_warp_kernel<T, R, INNER, KB>;
+  const int occ = occupancy(dev, kern, threads, 0);
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
   const int pm = prefetch_mode();
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
-  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
-                                              vec ? 1 : 0, region, pf);
+  kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
+                                           vec ? 1 : 0, pf);
   g_last_launches = 1;
   return cudaGetLastError();
+}
+
+// k >= log2 R: one register-path kernel for every such k; k < log2 R: the
+// blocked-inner kernel compiled for that k.
+template <typename T, int R, int INNER>
+cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                        int64_t S, int k, bool vec, cudaStream_t st) {
+  constexpr int LR = ilog2c(R);
+  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st);
+  switch (k) {
+    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st);
+    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st); break;
+    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st); break;
+    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st); break;
+  }
+  return cudaErrorInvalidValue;
 }
 
 template <typename T, int R, int W, int INNER>
@@ -181,7 +191,9 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
       case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
       case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
       case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 16: return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 16:
+        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+        break;
     }
     return cudaErrorInvalidValue;
   }

@@ -24,58 +24,34 @@ namespace tdg {
 // ============================================================================
 // Warp kernel.
 // ============================================================================
-template <typename T, int R, int INNER, bool SMEM>
+// KB < 0: k >= LR (all in-lane levels; m <= P, lane-level inner solve).
+// KB >= 0: k == KB < LR (m = P * (R >> KB) > P, register-blocked inner solve).
+template <typename T, int R, int INNER, int KB>
 __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&d)[R], int k,
-                                           int ls, int P, T* region) {
+                                           int ls, int P) {
   constexpr int LR = ilog2c(R);
-  // SMEM == false: k >= LR (all in-lane levels, m <= P); compile-time kin.
-  const int kin = SMEM ? (k < LR ? k : LR) : LR;
+  constexpr int kin = KB < 0 ? LR : KB;
   inlane_forward_interior<T, R>(a, b, c, d, kin);
   Heads<T, R> H;
   heads_from_next_lane<T, R>(a, b, c, d, kin, P, ls == P - 1, H);
   inlane_tail_chain<T, R>(a, b, c, d, kin, H);
-  if constexpr (!SMEM) {
+  if constexpr (KB < 0) {
     d[R - 1] = lane_level_solve<T, INNER>(a[R - 1], b[R - 1], c[R - 1], d[R - 1], k - LR, ls, P);
   } else {
-    // m = P * q > P: the q = R >> k survivors of each lane go to shared memory
-    // as a contiguous m-system (the paper's copy step).
-    const int q = R >> k;
-    const int m = P * q;
-    const int mask = (1 << k) - 1;
-    T* X = region + (INNER == kPCR ? 8 * m : 12 * m);
-#pragma unroll
-    for (int t = 0; t < R; ++t) {
-      if (((t + 1) & mask) == 0) {
-        const int j = ls * q + ((t + 1) >> k) - 1;
-        if constexpr (INNER == kPCR) {
-          region[j] = a[t]; region[m + j] = b[t]; region[2 * m + j] = c[t]; region[3 * m + j] = d[t];
-        } else {
-          rd_setup(a[t], b[t], c[t], d[t], j, m, region + j, m);
-        }
-      }
-    }
-    __syncwarp();
-    if constexpr (INNER == kPCR) smem_pcr<T>(region, X, m, ls, P, SyncWarp());
-    else smem_rd<T>(region, X, m, ls, P, SyncWarp());
-#pragma unroll
-    for (int t = 0; t < R; ++t) {
-      if (((t + 1) & mask) == 0) d[t] = X[ls * q + ((t + 1) >> k) - 1];
-    }
-    __syncwarp();
+    // m = P * (R >> KB) > P: the intermediate system stays block-distributed
+    // in registers (no copy; the paper copies it to 5 extra arrays).
+    if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
+    else blocked_rd<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
   }
   T xprev = __shfl_up_sync(kFull, d[R - 1], 1, P);
   if (ls == 0) xprev = T(0);
   inlane_backward<T, R>(a, b, c, d, kin, xprev);
 }
 
-// region_elems: shared-memory elements per system (0 when m <= P).
-template <typename T, int R, int INNER, bool SMEM>
+template <typename T, int R, int INNER, int KB>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                const T* d, T* x, int n, long long S, int k, int log2P, int vec,
-                int region_elems, int pf) {
-  extern __shared__ __align__(16) unsigned char smem_raw[];
-  T* smem = reinterpret_cast<T*>(smem_raw);
+                const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf) {
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -83,7 +59,6 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
   const int G = 32 >> log2P;  // systems per warp
   const int sub = lane >> log2P;
   const int ls = lane & (P - 1);
-  T* region = smem + (size_t)(warp * G + sub) * region_elems;
   const long long step = (long long)gridDim.x * wpb * G;
   for (long long s0 = ((long long)blockIdx.x * wpb + warp) * G; s0 < S; s0 += step) {
     if (pf && lane < 4 && s0 + step < S) {
@@ -109,7 +84,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
-    warp_solve<T, R, INNER, SMEM>(ra, rb, rc, rd, k, ls, P, region);
+    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
     if (valid) store_block<T, R>(x + off, rd, vec);
   }
 }
