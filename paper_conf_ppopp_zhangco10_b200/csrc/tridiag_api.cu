@@ -71,18 +71,27 @@ int g_force_R = -1, g_prefetch = -1;
 int force_R() { if (g_force_R < 0) g_force_R = env_int("TRIDIAG_WARP_R", 0); return g_force_R; }
 int prefetch_mode() { if (g_prefetch < 0) g_prefetch = env_int("TRIDIAG_PREFETCH", 2); return g_prefetch; }
 
-// R per lane from the plan sweep (profiles/r01_tune_plan.md): the widest
-// register block that fits (16 fp32 / 8 fp64 equations per lane) is fastest at
-// every n; systems with n <= 32 use 4 lanes (or n lanes when n < 4).
-Plan plan_for(int dtype, int64_t n) {
+// R per lane from the plan sweep (profiles/r01_tune_plan.md): on HBM-scale
+// batches the widest register block that fits (16 fp32 / 8 fp64 equations per
+// lane) is fastest at every n, and systems with n <= 32 use 4 lanes.  Small
+// batches (fewer than ~8 warps' worth of lanes per SM at that R) are latency
+// bound instead: they spread each system over more lanes (R = n/32, a full
+// warp), which keeps m <= 32 on the register path.  num_systems < 0 asks for
+// the HBM-scale plan.
+constexpr int64_t kSmallBatchLanes = 148LL * 8 * 32;
+
+Plan plan_for(int dtype, int64_t n, int64_t S = -1) {
   const int fr = force_R();
   const int Rmax = dtype == TRIDIAG_F32 ? 16 : 8;
   if (fr > 0 && fr <= Rmax && fr <= n && n / fr <= 32 && (fr & (fr - 1)) == 0) return {false, fr, 0};
-  if (n <= 32) return {false, (int)std::max<int64_t>(1, n / 4), 0};
-  if (n <= 32 * Rmax) return {false, Rmax, 0};
-  return {true, Rmax, (int)(n / (Rmax * 32))};
+  if (n > 32 * Rmax) return {true, Rmax, (int)(n / (Rmax * 32))};
+  int R = n <= 32 ? (int)std::max<int64_t>(1, n / 4) : Rmax;
+  if (S >= 0 && S * n / R < kSmallBatchLanes) R = (int)std::max<int64_t>(1, n / 32);
+  return {false, R, 0};
 }
 
+// Lanes per system of the HBM-scale plan: the largest m the hybrids keep on
+// the register path (the small-batch plan has at least as many lanes).
 int lanes_per_system(int dtype, int64_t n) {
   const Plan p = plan_for(dtype, n);
   return p.cta ? 32 : (int)(n / p.R);
@@ -181,7 +190,7 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
   const T* c = static_cast<const T*>(c_);
   const T* d = static_cast<const T*>(d_);
   T* x = static_cast<T*>(x_);
-  const Plan p = plan_for(dtype, n);
+  const Plan p = plan_for(dtype, n, S);
   const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
   auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
   const bool vec = al(a) && al(b) && al(c) && al(d) && al(x);

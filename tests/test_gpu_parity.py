@@ -277,6 +277,21 @@ def test_deterministic_and_partition_invariant():
             assert torch.equal(torch.cat(parts).view(torch.int8), x1.view(torch.int8))
 
 
+def test_small_batch_plan_is_bitwise_identical():
+    """Small batches spread a system over more lanes (latency-bound plan); the
+    arithmetic per equation is the same CR unit, so a system's x must not
+    depend on the batch it was solved in (partition invariance, R22)."""
+    for dtype in (torch.float32, torch.float64):
+        for n in [8, 32, 64, 128, 256]:
+            S = 60000
+            a, b, c, d = gen("dd", S, n, dtype)
+            for algo in ["cr", "cr_pcr", "cr_rd", "pcr", "rd"]:
+                big = gpu_solve(a, b, c, d, algo)
+                small = gpu_solve(a[:50].contiguous(), b[:50].contiguous(), c[:50].contiguous(),
+                                  d[:50].contiguous(), algo)
+                assert torch.equal(big[:50].view(torch.int8), small.view(torch.int8)), (dtype, n, algo)
+
+
 def test_hybrid_endpoints_bitwise():
     """Fig 17: CR+PCR(m=2) == CR, CR+PCR(m=n) == PCR,
     CR+RD(m=n) == RD, bitwise (NaN-safe: compare bit patterns)."""
