@@ -163,78 +163,97 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
 
     T xprev;
     if constexpr (!SMEM) {
-      // ---- P survivors (one per lane) -> compacted CR levels in smem ----
-      const int kr = k - LR;                 // CR levels left
-      const int m = P >> kr;                 // intermediate size
-      const int mt = m > 32 ? m : 32;        // reduce in smem down to mt
-      const int kmid = ilog2c(P) - ilog2c(mt);
-      T* LA = work;
-      T* LB = LA + 2 * P;
-      T* LC = LB + 2 * P;
-      T* LD = LC + 2 * P;
-      T* LX = LD + 2 * P;
-      T* inner = LX + 2 * P;
-      LA[ls] = ra[R - 1]; LB[ls] = rb[R - 1]; LC[ls] = rc[R - 1]; LD[ls] = rd[R - 1];
-      __syncthreads();
-      int offp = 0;  // offset of level l-1
-      for (int l = 1; l <= kmid; ++l) {
-        const int np = P >> (l - 1);  // equations at level l-1
-        const int offn = offp + np;   // offset of level l
-        const int j = ls;
-        if (j < (np >> 1)) {
-          const int i = offp + 2 * j + 1, lo = i - 1, hi = i + 1;
-          T ai = LA[i], bi = LB[i], ci = LC[i], di = LD[i];
-          const T rl = Arith<T>::rcp(LB[lo]);
-          T ha = T(0), hr = T(0), hc = T(0), hd = T(0);
-          if (2 * j + 2 < np) { ha = LA[hi]; hr = Arith<T>::rcp(LB[hi]); hc = LC[hi]; hd = LD[hi]; }
-          cr_unit(ai, bi, ci, di, LA[lo], rl, LC[lo], LD[lo], ha, hr, hc, hd);
-          LA[offn + j] = ai; LB[offn + j] = bi; LC[offn + j] = ci; LD[offn + j] = di;
+      // ---- lane-level CR inside every warp (shuffles), kl levels ----
+      const int kr = k - LR;                 // CR levels left after the in-lane ones
+      const int kl = kr < 5 ? kr : 5;        // of which across the lanes of a warp
+      T A = ra[R - 1], B = rb[R - 1], C = rc[R - 1], D = rd[R - 1];
+      // interior: every update lane except the warp's tail (lane 31)
+#pragma unroll
+      for (int l = 1; l <= 5; ++l) {
+        if (l <= kl) {
+          const int sg = 1 << (l - 1);
+          const int md = lane & (2 * sg - 1);
+          if (md == sg - 1) B = Arith<T>::rcp(B);
+          const T la = shup(A, sg, 32), lb = shup(B, sg, 32), lc = shup(C, sg, 32), ld = shup(D, sg, 32);
+          const T ha = shdn(A, sg, 32), hb = shdn(B, sg, 32), hc = shdn(C, sg, 32), hd = shdn(D, sg, 32);
+          if (md == 2 * sg - 1 && lane != 31) cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
         }
-        __syncthreads();
-        offp = offn;
       }
-      // level kmid (mt equations) at offset offp
-      if (m <= 32) {
+      // lane heads of warp w (lanes 2^(l-1)-1, final state) for warp w-1's tail
+      T* heads2 = heads + W * LRH * 4;                 // [W][5][4]
+      T* surv = heads2 + W * 5 * 4;                    // [4][P] survivors (m_surv <= 32)
+      T* xs = surv + 4 * P;                            // [P]
+      T* inner = xs + P;                               // inner region (m_surv > 32)
+      if (warp > 0 && ((lane + 1) & lane) == 0 && lane < (1 << kl)) {
+        const int l = ilog2c(lane + 1);               // lane = 2^l - 1 -> level l+1
+        T* hp = heads2 + (warp * 5 + l) * 4;
+        hp[0] = A; hp[1] = B; hp[2] = C; hp[3] = D;
+      }
+      __syncthreads();
+      // tail chain of lane 31: lower neighbour lane 31-sg (final), upper = next warp's head
+#pragma unroll
+      for (int l = 1; l <= 5; ++l) {
+        if (l <= kl) {
+          const int sg = 1 << (l - 1);
+          const T la = __shfl_sync(kFull, A, 31 - sg), lb = __shfl_sync(kFull, B, 31 - sg);
+          const T lc = __shfl_sync(kFull, C, 31 - sg), ld = __shfl_sync(kFull, D, 31 - sg);
+          if (lane == 31) {
+            T ha = T(0), hb = T(0), hc = T(0), hd = T(0);
+            if (warp + 1 < W) {
+              const T* hp = heads2 + ((warp + 1) * 5 + (l - 1)) * 4;
+              ha = hp[0]; hb = hp[1]; hc = hp[2]; hd = hp[3];
+            }
+            cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
+          }
+        }
+      }
+      // survivors: lanes 2^kl - 1 (mod 2^kl) of every warp
+      const int per_warp = 32 >> kl;
+      const int msurv = W * per_warp;
+      const bool is_surv = ((lane + 1) & ((1 << kl) - 1)) == 0;
+      const int j = warp * per_warp + (lane >> kl);
+      if (msurv <= 32) {
+        if (is_surv) { surv[j] = A; surv[P + j] = B; surv[2 * P + j] = C; surv[3 * P + j] = D; }
+      } else if (is_surv) {
+        // kl == kr: the survivors are the m-system; shared-memory inner on the CTA
+        if constexpr (INNER == kPCR) {
+          inner[j] = A; inner[msurv + j] = B; inner[2 * msurv + j] = C; inner[3 * msurv + j] = D;
+        } else {
+          rd_setup(A, B, C, D, j, msurv, inner + j, msurv);
+        }
+      }
+      __syncthreads();
+      if (msurv <= 32) {
         if (warp == 0) {
-          const T X = lane_level_solve<T, INNER>(LA[offp + lane], LB[offp + lane],
-                                                 LC[offp + lane], LD[offp + lane],
-                                                 ilog2c(32) - ilog2c(m), lane, 32);
-          LX[offp + lane] = X;
+          const bool v = lane < msurv;
+          const T sA = v ? surv[lane] : T(0), sB = v ? surv[P + lane] : T(1);
+          const T sC = v ? surv[2 * P + lane] : T(0), sD = v ? surv[3 * P + lane] : T(0);
+          const T X = lane_level_solve<T, INNER>(sA, sB, sC, sD, kr - kl, lane & (msurv - 1), msurv);
+          if (v) xs[lane] = X;
         }
       } else {
-        if constexpr (INNER == kPCR) {
-          for (int j = ls; j < m; j += P) {
-            inner[j] = LA[offp + j]; inner[m + j] = LB[offp + j];
-            inner[2 * m + j] = LC[offp + j]; inner[3 * m + j] = LD[offp + j];
-          }
-        } else {
-          for (int j = ls; j < m; j += P)
-            rd_setup(LA[offp + j], LB[offp + j], LC[offp + j], LD[offp + j], j, m, inner + j, m);
-        }
-        __syncthreads();
-        T* X = inner + (INNER == kPCR ? 8 * m : 12 * m);
-        if constexpr (INNER == kPCR) smem_pcr<T>(inner, X, m, ls, P, SyncCta());
-        else smem_rd<T>(inner, X, m, ls, P, SyncCta());
-        for (int j = ls; j < m; j += P) LX[offp + j] = X[j];
+        if constexpr (INNER == kPCR) smem_pcr<T>(inner, xs, msurv, ls, P, SyncCta());
+        else smem_rd<T>(inner, xs, msurv, ls, P, SyncCta());
       }
       __syncthreads();
-      // backward through the compacted levels: level l-1 from level l
-      for (int l = kmid; l >= 1; --l) {
-        const int np = P >> (l - 1);
-        const int offl = 2 * P - 2 * (P >> l);       // level l
-        const int offm = 2 * P - 2 * np;             // level l-1
-        const int j = ls;
-        if (j < (np >> 1)) {
-          const T xo = LX[offl + j];                  // x of equation 2j+1 of level l-1
-          const T xl = (j > 0) ? LX[offl + j - 1] : T(0);
-          const int e = offm + 2 * j;
-          LX[e] = Arith<T>::div(LD[e] - LA[e] * xl - LC[e] * xo, LB[e]);
-          LX[e + 1] = xo;
+      // lane-level backward inside the warp
+      const T xprev_warp = warp > 0 ? xs[warp * per_warp - 1] : T(0);
+      T X = is_surv ? xs[j] : T(0);
+#pragma unroll
+      for (int l = 5; l >= 1; --l) {
+        if (l <= kl) {
+          const int sg = 1 << (l - 1);
+          T xl = shup(X, sg, 32);
+          const T xh = shdn(X, sg, 32);
+          if ((lane & (2 * sg - 1)) == sg - 1) {
+            if (lane < sg) xl = xprev_warp;
+            X = back_unit(A, B, C, D, xl, xh);
+          }
         }
-        __syncthreads();
       }
-      rd[R - 1] = LX[ls];
-      xprev = ls > 0 ? LX[ls - 1] : T(0);
+      rd[R - 1] = X;
+      const T xup = shup(X, 1, 32);
+      xprev = lane > 0 ? xup : xprev_warp;
     } else {
       // ---- m = P * q > P: shared-memory inner on the whole CTA ----
       const int q = R >> k;
@@ -276,9 +295,11 @@ inline size_t cta_smem_bytes(int R, int W, int inner, int k) {
   const int LRH = LR > 0 ? LR : 1;
   int64_t e = (int64_t)W * LRH * 4;
   if (k >= LR) {
-    const int m = P >> (k - LR);
-    e += 10LL * P;
-    if (m > 32) e += inner_region_elems(inner, m);
+    const int kr = k - LR;
+    const int kl = kr < 5 ? kr : 5;
+    const int64_t msurv = (int64_t)W * (32 >> kl);
+    e += (int64_t)W * 5 * 4 + 4LL * P + P;
+    if (msurv > 32) e += inner_region_elems(inner, msurv);
   } else {
     const int64_t m = (int64_t)P * (R >> k);
     e += inner_region_elems(inner, m);
