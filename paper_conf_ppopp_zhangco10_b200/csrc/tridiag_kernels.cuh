@@ -184,7 +184,7 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       T* surv = heads2 + W * 5 * 4;                    // [4][P] survivors (m_surv <= 32)
       T* xs = surv + 4 * P;                            // [P]
       T* inner = xs + P;                               // inner region (m_surv > 32)
-      if (warp > 0 && ((lane + 1) & lane) == 0 && lane < (1 << kl)) {
+      if (warp > 0 && ((lane + 1) & lane) == 0 && lane < (1 << (kl - 1))) {
         const int l = ilog2c(lane + 1);               // lane = 2^l - 1 -> level l+1
         T* hp = heads2 + (warp * 5 + l) * 4;
         hp[0] = A; hp[1] = B; hp[2] = C; hp[3] = D;
