@@ -12,7 +12,9 @@
 #include <tuple>
 
 #include "tridiag.h"
-#include "tridiag_kernels.cuh"
+#include "tridiag_tma.cuh"
+
+#include <cudaTypedefs.h>
 
 namespace {
 
@@ -164,9 +166,74 @@ cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, in
   return cudaErrorInvalidValue;
 }
 
+// ---------------------------------------------------------------------------
+// TMA tensor maps (driver entry point fetched once through the runtime).
+// ---------------------------------------------------------------------------
+PFN_cuTensorMapEncodeTiled_v12000 encode_fn() {
+  static PFN_cuTensorMapEncodeTiled_v12000 fn = nullptr;
+  static std::once_flag once;
+  std::call_once(once, [] {
+    void* p = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      fn = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
+  });
+  return fn;
+}
+
+// View one input array as [S*n/R rows][R columns] (64-byte rows), boxes of
+// min(P, 256) rows, 64-byte swizzle.
+template <typename T>
+bool make_row_map(CUtensorMap* m, const void* base, int64_t rows, int R, int box_rows) {
+  auto fn = encode_fn();
+  if (!fn) return false;
+  const cuuint64_t dims[2] = {(cuuint64_t)R, (cuuint64_t)rows};
+  const cuuint64_t strides[1] = {(cuuint64_t)R * sizeof(T)};
+  const cuuint32_t box[2] = {(cuuint32_t)R, (cuuint32_t)box_rows};
+  const cuuint32_t estr[2] = {1, 1};
+  const CUresult r = fn(m, sizeof(T) == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64,
+                        2, const_cast<void*>(base), dims, strides, box, estr,
+                        CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_64B,
+                        CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS;
+}
+
+template <typename T, int R, int W, int INNER>
+cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                           int64_t S, int k, cudaStream_t st, bool* used) {
+  *used = false;
+  const int P = 32 * W;
+  const int64_t rows = S * P;
+  if (rows >= (int64_t(1) << 31)) return cudaSuccess;
+  CUtensorMap mA, mB, mC, mD;
+  const int box = P > 256 ? 256 : P;
+  if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
+      !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box))
+    return cudaSuccess;
+  const size_t smem = tdg::cta_tma_smem_bytes<T>(R, W, INNER, k);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER>;
+  const int occ = occupancy(dev, kern, W * 32, smem);
+  if (occ <= 0) return cudaSuccess;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(mA, mB, mC, mD, x, (int)n, (long long)S, k);
+  g_last_launches = 1;
+  *used = true;
+  return cudaGetLastError();
+}
+
+int tma_mode() { static int v = env_int("TRIDIAG_TMA", 1); return v; }
+
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
                        int64_t S, int k, bool vec, cudaStream_t st) {
+  if (vec && k >= ilog2c(R) && tma_mode()) {
+    bool used = false;
+    const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
+    if (used || e != cudaSuccess) return e;
+  }
   const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k);
   int dev = 0;
   cudaGetDevice(&dev);

@@ -98,6 +98,160 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 //                  + inner region for m > 32
 //   case k <  LR:  inner region for m = P * (R >> k)
 // ============================================================================
+// In-lane CR (heads of the next warp through shared memory, one barrier) for
+// a CTA that owns one system; AfterB1 runs right after that barrier (the TMA
+// kernel issues the next system's copy there: every thread has consumed its
+// staged input by then).
+template <typename T, int R, int W, class AfterB1>
+__device__ __forceinline__ void cta_inlane_forward(T (&ra)[R], T (&rb)[R], T (&rc)[R], T (&rd)[R],
+                                                   int kin, T* heads, AfterB1 after_b1) {
+  constexpr int LR = ilog2c(R);
+  constexpr int LRH = LR > 0 ? LR : 1;
+  const int ls = threadIdx.x;
+  const int lane = ls & 31;
+  const int warp = ls >> 5;
+    inlane_forward_interior<T, R>(ra, rb, rc, rd, kin);
+    // Heads: lanes 0..30 take them from lane+1 by shuffle; lane 31 of warp w
+    // takes warp w+1's lane 0 through shared memory.
+    Heads<T, R> H;
+    heads_from_next_lane<T, R>(ra, rb, rc, rd, kin, 32, false, H);
+    if (lane == 0 && warp > 0) {
+#pragma unroll
+      for (int l = 1; l <= LR; ++l) {
+        if (l <= kin) {
+          const int t = (1 << (l - 1)) - 1;
+          T* hp = heads + (warp * LRH + (l - 1)) * 4;
+          hp[0] = ra[t]; hp[1] = rb[t]; hp[2] = rc[t]; hp[3] = rd[t];
+        }
+      }
+    }
+    __syncthreads();
+    after_b1();
+    if (lane == 31) {
+#pragma unroll
+      for (int l = 1; l <= LR; ++l) {
+        if (l <= kin) {
+          if (warp + 1 < W) {
+            const T* hp = heads + ((warp + 1) * LRH + (l - 1)) * 4;
+            H.a[l - 1] = hp[0]; H.rb[l - 1] = hp[1]; H.c[l - 1] = hp[2]; H.d[l - 1] = hp[3];
+          } else {
+            H.a[l - 1] = T(0); H.rb[l - 1] = T(0); H.c[l - 1] = T(0); H.d[l - 1] = T(0);
+          }
+        }
+      }
+    }
+    inlane_tail_chain<T, R>(ra, rb, rc, rd, kin, H);
+
+}
+
+// Register path (k >= log2 R, m <= 32 lanes or m = survivors): lane-level CR
+// inside every warp, survivors solved by one warp or by the CTA in shared
+// memory, back-substitution.  Returns xprev for the in-lane back-substitution
+// and leaves x of the lane's tail in rd[R-1].
+template <typename T, int R, int W, int INNER>
+__device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R], T (&rd)[R],
+                                               int k, T* heads) {
+  constexpr int P = 32 * W;
+  constexpr int LR = ilog2c(R);
+  constexpr int LRH = LR > 0 ? LR : 1;
+  const int ls = threadIdx.x;
+  const int lane = ls & 31;
+  const int warp = ls >> 5;
+  T xprev;
+    // ---- lane-level CR inside every warp (shuffles), kl levels ----
+    const int kr = k - LR;                 // CR levels left after the in-lane ones
+    const int kl = kr < 5 ? kr : 5;        // of which across the lanes of a warp
+    T A = ra[R - 1], B = rb[R - 1], C = rc[R - 1], D = rd[R - 1];
+    // interior: every update lane except the warp's tail (lane 31)
+#pragma unroll
+    for (int l = 1; l <= 5; ++l) {
+      if (l <= kl) {
+        const int sg = 1 << (l - 1);
+        const int md = lane & (2 * sg - 1);
+        if (md == sg - 1) B = Arith<T>::rcp(B);
+        const T la = shup(A, sg, 32), lb = shup(B, sg, 32), lc = shup(C, sg, 32), ld = shup(D, sg, 32);
+        const T ha = shdn(A, sg, 32), hb = shdn(B, sg, 32), hc = shdn(C, sg, 32), hd = shdn(D, sg, 32);
+        if (md == 2 * sg - 1 && lane != 31) cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
+      }
+    }
+    // lane heads of warp w (lanes 2^(l-1)-1, final state) for warp w-1's tail
+    T* heads2 = heads + W * LRH * 4;                 // [W][5][4]
+    T* surv = heads2 + W * 5 * 4;                    // [4][P] survivors (m_surv <= 32)
+    T* xs = surv + 4 * P;                            // [P]
+    T* inner = xs + P;                               // inner region (m_surv > 32)
+    if (warp > 0 && ((lane + 1) & lane) == 0 && lane < (1 << (kl - 1))) {
+      const int l = ilog2c(lane + 1);               // lane = 2^l - 1 -> level l+1
+      T* hp = heads2 + (warp * 5 + l) * 4;
+      hp[0] = A; hp[1] = B; hp[2] = C; hp[3] = D;
+    }
+    __syncthreads();
+    // tail chain of lane 31: lower neighbour lane 31-sg (final), upper = next warp's head
+#pragma unroll
+    for (int l = 1; l <= 5; ++l) {
+      if (l <= kl) {
+        const int sg = 1 << (l - 1);
+        const T la = __shfl_sync(kFull, A, 31 - sg), lb = __shfl_sync(kFull, B, 31 - sg);
+        const T lc = __shfl_sync(kFull, C, 31 - sg), ld = __shfl_sync(kFull, D, 31 - sg);
+        if (lane == 31) {
+          T ha = T(0), hb = T(0), hc = T(0), hd = T(0);
+          if (warp + 1 < W) {
+            const T* hp = heads2 + ((warp + 1) * 5 + (l - 1)) * 4;
+            ha = hp[0]; hb = hp[1]; hc = hp[2]; hd = hp[3];
+          }
+          cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
+        }
+      }
+    }
+    // survivors: lanes 2^kl - 1 (mod 2^kl) of every warp
+    const int per_warp = 32 >> kl;
+    const int msurv = W * per_warp;
+    const bool is_surv = ((lane + 1) & ((1 << kl) - 1)) == 0;
+    const int j = warp * per_warp + (lane >> kl);
+    if (msurv <= 32) {
+      if (is_surv) { surv[j] = A; surv[P + j] = B; surv[2 * P + j] = C; surv[3 * P + j] = D; }
+    } else if (is_surv) {
+      // kl == kr: the survivors are the m-system; shared-memory inner on the CTA
+      if constexpr (INNER == kPCR) {
+        inner[j] = A; inner[msurv + j] = B; inner[2 * msurv + j] = C; inner[3 * msurv + j] = D;
+      } else {
+        rd_setup(A, B, C, D, j, msurv, inner + j, msurv);
+      }
+    }
+    __syncthreads();
+    if (msurv <= 32) {
+      if (warp == 0) {
+        const bool v = lane < msurv;
+        const T sA = v ? surv[lane] : T(0), sB = v ? surv[P + lane] : T(1);
+        const T sC = v ? surv[2 * P + lane] : T(0), sD = v ? surv[3 * P + lane] : T(0);
+        const T X = lane_level_solve<T, INNER>(sA, sB, sC, sD, kr - kl, lane & (msurv - 1), msurv);
+        if (v) xs[lane] = X;
+      }
+    } else {
+      if constexpr (INNER == kPCR) smem_pcr<T>(inner, xs, msurv, ls, P, SyncCta());
+      else smem_rd<T>(inner, xs, msurv, ls, P, SyncCta());
+    }
+    __syncthreads();
+    // lane-level backward inside the warp
+    const T xprev_warp = warp > 0 ? xs[warp * per_warp - 1] : T(0);
+    T X = is_surv ? xs[j] : T(0);
+#pragma unroll
+    for (int l = 5; l >= 1; --l) {
+      if (l <= kl) {
+        const int sg = 1 << (l - 1);
+        T xl = shup(X, sg, 32);
+        const T xh = shdn(X, sg, 32);
+        if ((lane & (2 * sg - 1)) == sg - 1) {
+          if (lane < sg) xl = xprev_warp;
+          X = back_unit(A, B, C, D, xl, xh);
+        }
+      }
+    }
+    rd[R - 1] = X;
+    const T xup = shup(X, 1, 32);
+    xprev = lane > 0 ? xup : xprev_warp;
+  return xprev;
+}
+
 template <typename T, int R, int W, int INNER, bool SMEM>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
@@ -130,130 +284,10 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
 
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, kin);
-    // Heads: lanes 0..30 take them from lane+1 by shuffle; lane 31 of warp w
-    // takes warp w+1's lane 0 through shared memory.
-    Heads<T, R> H;
-    heads_from_next_lane<T, R>(ra, rb, rc, rd, kin, 32, false, H);
-    if (lane == 0 && warp > 0) {
-#pragma unroll
-      for (int l = 1; l <= LR; ++l) {
-        if (l <= kin) {
-          const int t = (1 << (l - 1)) - 1;
-          T* hp = heads + (warp * LRH + (l - 1)) * 4;
-          hp[0] = ra[t]; hp[1] = rb[t]; hp[2] = rc[t]; hp[3] = rd[t];
-        }
-      }
-    }
-    __syncthreads();
-    if (lane == 31) {
-#pragma unroll
-      for (int l = 1; l <= LR; ++l) {
-        if (l <= kin) {
-          if (warp + 1 < W) {
-            const T* hp = heads + ((warp + 1) * LRH + (l - 1)) * 4;
-            H.a[l - 1] = hp[0]; H.rb[l - 1] = hp[1]; H.c[l - 1] = hp[2]; H.d[l - 1] = hp[3];
-          } else {
-            H.a[l - 1] = T(0); H.rb[l - 1] = T(0); H.c[l - 1] = T(0); H.d[l - 1] = T(0);
-          }
-        }
-      }
-    }
-    inlane_tail_chain<T, R>(ra, rb, rc, rd, kin, H);
-
+    cta_inlane_forward<T, R, W>(ra, rb, rc, rd, kin, heads, [] {});
     T xprev;
     if constexpr (!SMEM) {
-      // ---- lane-level CR inside every warp (shuffles), kl levels ----
-      const int kr = k - LR;                 // CR levels left after the in-lane ones
-      const int kl = kr < 5 ? kr : 5;        // of which across the lanes of a warp
-      T A = ra[R - 1], B = rb[R - 1], C = rc[R - 1], D = rd[R - 1];
-      // interior: every update lane except the warp's tail (lane 31)
-#pragma unroll
-      for (int l = 1; l <= 5; ++l) {
-        if (l <= kl) {
-          const int sg = 1 << (l - 1);
-          const int md = lane & (2 * sg - 1);
-          if (md == sg - 1) B = Arith<T>::rcp(B);
-          const T la = shup(A, sg, 32), lb = shup(B, sg, 32), lc = shup(C, sg, 32), ld = shup(D, sg, 32);
-          const T ha = shdn(A, sg, 32), hb = shdn(B, sg, 32), hc = shdn(C, sg, 32), hd = shdn(D, sg, 32);
-          if (md == 2 * sg - 1 && lane != 31) cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
-        }
-      }
-      // lane heads of warp w (lanes 2^(l-1)-1, final state) for warp w-1's tail
-      T* heads2 = heads + W * LRH * 4;                 // [W][5][4]
-      T* surv = heads2 + W * 5 * 4;                    // [4][P] survivors (m_surv <= 32)
-      T* xs = surv + 4 * P;                            // [P]
-      T* inner = xs + P;                               // inner region (m_surv > 32)
-      if (warp > 0 && ((lane + 1) & lane) == 0 && lane < (1 << (kl - 1))) {
-        const int l = ilog2c(lane + 1);               // lane = 2^l - 1 -> level l+1
-        T* hp = heads2 + (warp * 5 + l) * 4;
-        hp[0] = A; hp[1] = B; hp[2] = C; hp[3] = D;
-      }
-      __syncthreads();
-      // tail chain of lane 31: lower neighbour lane 31-sg (final), upper = next warp's head
-#pragma unroll
-      for (int l = 1; l <= 5; ++l) {
-        if (l <= kl) {
-          const int sg = 1 << (l - 1);
-          const T la = __shfl_sync(kFull, A, 31 - sg), lb = __shfl_sync(kFull, B, 31 - sg);
-          const T lc = __shfl_sync(kFull, C, 31 - sg), ld = __shfl_sync(kFull, D, 31 - sg);
-          if (lane == 31) {
-            T ha = T(0), hb = T(0), hc = T(0), hd = T(0);
-            if (warp + 1 < W) {
-              const T* hp = heads2 + ((warp + 1) * 5 + (l - 1)) * 4;
-              ha = hp[0]; hb = hp[1]; hc = hp[2]; hd = hp[3];
-            }
-            cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
-          }
-        }
-      }
-      // survivors: lanes 2^kl - 1 (mod 2^kl) of every warp
-      const int per_warp = 32 >> kl;
-      const int msurv = W * per_warp;
-      const bool is_surv = ((lane + 1) & ((1 << kl) - 1)) == 0;
-      const int j = warp * per_warp + (lane >> kl);
-      if (msurv <= 32) {
-        if (is_surv) { surv[j] = A; surv[P + j] = B; surv[2 * P + j] = C; surv[3 * P + j] = D; }
-      } else if (is_surv) {
-        // kl == kr: the survivors are the m-system; shared-memory inner on the CTA
-        if constexpr (INNER == kPCR) {
-          inner[j] = A; inner[msurv + j] = B; inner[2 * msurv + j] = C; inner[3 * msurv + j] = D;
-        } else {
-          rd_setup(A, B, C, D, j, msurv, inner + j, msurv);
-        }
-      }
-      __syncthreads();
-      if (msurv <= 32) {
-        if (warp == 0) {
-          const bool v = lane < msurv;
-          const T sA = v ? surv[lane] : T(0), sB = v ? surv[P + lane] : T(1);
-          const T sC = v ? surv[2 * P + lane] : T(0), sD = v ? surv[3 * P + lane] : T(0);
-          const T X = lane_level_solve<T, INNER>(sA, sB, sC, sD, kr - kl, lane & (msurv - 1), msurv);
-          if (v) xs[lane] = X;
-        }
-      } else {
-        if constexpr (INNER == kPCR) smem_pcr<T>(inner, xs, msurv, ls, P, SyncCta());
-        else smem_rd<T>(inner, xs, msurv, ls, P, SyncCta());
-      }
-      __syncthreads();
-      // lane-level backward inside the warp
-      const T xprev_warp = warp > 0 ? xs[warp * per_warp - 1] : T(0);
-      T X = is_surv ? xs[j] : T(0);
-#pragma unroll
-      for (int l = 5; l >= 1; --l) {
-        if (l <= kl) {
-          const int sg = 1 << (l - 1);
-          T xl = shup(X, sg, 32);
-          const T xh = shdn(X, sg, 32);
-          if ((lane & (2 * sg - 1)) == sg - 1) {
-            if (lane < sg) xl = xprev_warp;
-            X = back_unit(A, B, C, D, xl, xh);
-          }
-        }
-      }
-      rd[R - 1] = X;
-      const T xup = shup(X, 1, 32);
-      xprev = lane > 0 ? xup : xprev_warp;
+      xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
     } else {
       // ---- m = P * q > P: shared-memory inner on the whole CTA ----
       const int q = R >> k;

@@ -1,0 +1,142 @@
+// tridiag_tma.cuh -- TMA-pipelined CTA kernel for large systems (sm_100a).
+//
+// One CTA owns one system at a time (W warps, R equations per lane, as in
+// tdg_cta_kernel).  Its four input arrays arrive through the Tensor Memory
+// Accelerator: each array is viewed as a 2-D tensor of 64-byte rows (one row =
+// one lane's R consecutive equations), copied with cp.async.bulk.tensor into a
+// shared-memory stage with the 64-byte swizzle, which makes the lane-blocked
+// 128-bit reads bank-conflict free (16-byte chunk q of row r sits at chunk
+// q ^ ((r >> 1) & 3)).  The copy of the NEXT system is issued as soon as every
+// thread has pulled the current one into registers, so HBM streams while the
+// CTA runs its CR levels (the paper's block-level overlap, made
+// explicit).  Completion is tracked by an mbarrier with expect-tx bytes.
+#pragma once
+
+#include <cuda.h>
+
+#include "tridiag_kernels.cuh"
+
+namespace tdg {
+
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+  asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+}
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)),
+               "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
+  uint32_t done = 0;
+  do {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n"
+        " selp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(done)
+        : "r"(smem_u32(bar)), "r"(parity)
+        : "memory");
+  } while (!done);
+}
+__device__ __forceinline__ void tma_load_2d(void* dst, const CUtensorMap* map, int c0, int c1,
+                                            uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::"r"(
+          smem_u32(dst)),
+      "l"(reinterpret_cast<uint64_t>(map)), "r"(c0), "r"(c1), "r"(smem_u32(bar))
+      : "memory");
+}
+
+// One lane's 64-byte row out of the 64B-swizzled stage: 16-byte chunk ch is
+// stored at chunk ch ^ sw, sw = (row >> 1) & 3 (CU_TENSOR_MAP_SWIZZLE_64B).
+template <typename T, int R>
+__device__ __forceinline__ void read_row(const unsigned char* row, int sw, T (&v)[R]) {
+  constexpr int E = 16 / (int)sizeof(T);
+#pragma unroll
+  for (int ch = 0; ch < 4; ++ch) {
+    const unsigned char* src = row + ((ch ^ sw) << 4);
+    if constexpr (sizeof(T) == 4) {
+      const float4 t = *reinterpret_cast<const float4*>(src);
+      v[ch * E + 0] = t.x; v[ch * E + 1] = t.y; v[ch * E + 2] = t.z; v[ch * E + 3] = t.w;
+    } else {
+      const double2 t = *reinterpret_cast<const double2*>(src);
+      v[ch * E + 0] = t.x; v[ch * E + 1] = t.y;
+    }
+  }
+}
+
+// Bytes of the TMA stage (a, b, c, d of one system), rounded to 1 KB.
+template <typename T>
+__host__ __device__ constexpr uint32_t tma_stage_bytes(int R, int W) {
+  return (uint32_t)(((4u * 32u * W * R * sizeof(T)) + 1023u) & ~1023u);
+}
+
+template <typename T, int R, int W, int INNER>
+__global__ void __launch_bounds__(W * 32)
+tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
+                   const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
+                   T* x, int n, long long S, int k) {
+  static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
+  constexpr int P = 32 * W;
+  constexpr int LR = ilog2c(R);
+  constexpr int ROWS = P > 256 ? 256 : P;  // rows per TMA box (box dims <= 256)
+  constexpr int NBOX = P / ROWS;
+  constexpr uint32_t ARR_BYTES = P * R * sizeof(T);
+  constexpr uint32_t STAGE = tma_stage_bytes<T>(R, W);
+  extern __shared__ __align__(1024) unsigned char smem_raw[];
+  unsigned char* stage = smem_raw;
+  uint64_t* bar = reinterpret_cast<uint64_t*>(smem_raw + STAGE);
+  T* heads = reinterpret_cast<T*>(smem_raw + STAGE + 16);
+  const int ls = threadIdx.x;
+
+  const CUtensorMap* maps[4] = {&tmA, &tmB, &tmC, &tmD};
+  auto issue = [&](long long sys) {
+    mbar_arrive_expect_tx(bar, 4 * ARR_BYTES);
+#pragma unroll
+    for (int q = 0; q < 4; ++q)
+#pragma unroll
+      for (int bx = 0; bx < NBOX; ++bx)
+        tma_load_2d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0,
+                    (int)(sys * P + bx * ROWS), bar);
+  };
+  if (ls == 0) {
+    mbar_init(bar, 1);
+    if (blockIdx.x < S) issue(blockIdx.x);
+  }
+  __syncthreads();
+
+  uint32_t parity = 0;
+  for (long long sys = blockIdx.x; sys < S; sys += gridDim.x) {
+    mbar_wait(bar, parity);
+    parity ^= 1;
+    T ra[R], rb[R], rc[R], rd[R];
+    const int sw = (ls >> 1) & 3;
+    read_row<T, R>(stage + 0 * ARR_BYTES + ls * 64, sw, ra);
+    read_row<T, R>(stage + 1 * ARR_BYTES + ls * 64, sw, rb);
+    read_row<T, R>(stage + 2 * ARR_BYTES + ls * 64, sw, rc);
+    read_row<T, R>(stage + 3 * ARR_BYTES + ls * 64, sw, rd);
+    if (ls == 0) ra[0] = T(0);
+    if (ls == P - 1) rc[R - 1] = T(0);
+    const long long next = sys + gridDim.x;
+    // every thread has read the stage once the heads barrier is passed
+    cta_inlane_forward<T, R, W>(ra, rb, rc, rd, LR, heads, [&] {
+      if (ls == 0 && next < S) issue(next);
+    });
+    const T xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
+    inlane_backward<T, R>(ra, rb, rc, rd, LR, xprev);
+    store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
+    __syncthreads();  // heads / survivor regions are reused by the next system
+  }
+}
+
+// Dynamic shared memory of tdg_cta_tma_kernel: stage + mbarrier + the
+// register path's regions (heads, lane heads, survivors, inner).
+template <typename T>
+inline size_t cta_tma_smem_bytes(int R, int W, int inner, int k) {
+  return tma_stage_bytes<T>(R, W) + 16 + cta_smem_bytes<T>(R, W, inner, k);
+}
+
+}  // namespace tdg
