@@ -44,8 +44,8 @@ typedef enum {
 enum {
     TRIDIAG_OK = 0,
     TRIDIAG_ERR_NULL = -1,         /* a pointer is NULL while num_systems > 0        */
-    TRIDIAG_ERR_N = -2,            /* n < 2 or n not a power of two     */
-    TRIDIAG_ERR_N_TOO_LARGE = -3,  /* n > tridiag_max_n(dtype, algo)                 */
+    TRIDIAG_ERR_N = -2,            /* n < 1                                          */
+    TRIDIAG_ERR_N_TOO_LARGE = -3,  /* next power of two of n > tridiag_max_n         */
     TRIDIAG_ERR_NUM_SYSTEMS = -4,  /* num_systems < 0                                */
     TRIDIAG_ERR_DTYPE = -5,        /* dtype not a tridiag_dtype                      */
     TRIDIAG_ERR_ALGO = -6,         /* algo not a tridiag_algo                        */
@@ -70,7 +70,12 @@ enum {
  * a, b, c, d  device pointers, read only.
  * x           device pointer, written.  x == d (exact in-place) is allowed;
  *             any other overlap of x with an input is TRIDIAG_ERR_OVERLAP.
- * n           equations per system: a power of two, 2 <= n <= tridiag_max_n.
+ * n           equations per system, n >= 1.  The paper's solvers take powers of
+ *             two; other n are solved as the next power of two
+ *             n_pad with padding equations x_i + c_pad x_{i+1} = 0 (i >= n,
+ *             solution 0; c_pad = 1 for the RD inner, which needs nonzero
+ *             c, else 0) and only the n real elements are read / written
+ *             (scalar-load path).  n_pad <= tridiag_max_n(dtype, algo).
  * num_systems S >= 0.  S == 0 returns TRIDIAG_OK without launching (the
  *             pointers may then be NULL; the other arguments are validated).
  * dtype       TRIDIAG_F32 or TRIDIAG_F64.  All arithmetic is in this type.
@@ -78,7 +83,7 @@ enum {
  * switch_level  the intermediate system size m of the hybrids (Fig 17's
  *             x-axis, "size-256 intermediate"): 0 = the tuned
  *             table (tridiag_auto_switch_level); else a power of two with
- *             2 <= m <= n and m <= tridiag_max_switch_level(dtype, algo, n).
+ *             2 <= m <= n_pad and m <= tridiag_max_switch_level(dtype, algo, n).
  *             m = 2 reproduces CR and m = n reproduces PCR / RD.  Must be 0
  *             for the non-hybrid algorithms.
  * stream      CUDA stream the work is enqueued on (asynchronous, no host

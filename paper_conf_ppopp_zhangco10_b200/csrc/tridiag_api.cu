@@ -23,6 +23,9 @@ using tdg::ilog2c;
 thread_local int g_last_launches = 0;
 
 bool is_pow2(int64_t v) { return v >= 1 && (v & (v - 1)) == 0; }
+// Systems are solved at the next power of two >= max(n, 2) (ragged n is padded
+// in the kernels, see load_ragged); everything below works on n_pad.
+int64_t pad_n(int64_t n) { int64_t p = 2; while (p < n) p <<= 1; return p; }
 int ilog2_64(int64_t v) { int l = 0; while ((int64_t(1) << l) < v) ++l; return l; }
 bool is_hybrid(int algo) { return algo == TRIDIAG_CR_PCR || algo == TRIDIAG_CR_RD; }
 size_t elem_size(int dtype) { return dtype == TRIDIAG_F64 ? 8 : 4; }
@@ -129,7 +132,7 @@ int occupancy(int dev, K kernel, int threads, size_t smem) {
 
 template <typename T, int R, int INNER, int KB>
 cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                          int64_t S, int k, bool vec, cudaStream_t st) {
+                          int64_t S, int k, bool vec, cudaStream_t st, int64_t n_real) {
   const int P = (int)(n / R);
   const int log2P = ilog2c(P);
   const int G = 32 / P;
@@ -144,8 +147,9 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
   const int pm = prefetch_mode();
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
-                                           vec ? 1 : 0, pf);
+                                           vec ? 1 : 0, pf, (int)n_real, c_pad);
   g_last_launches = 1;
   return cudaGetLastError();
 }
@@ -154,14 +158,14 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
 // blocked-inner kernel compiled for that k.
 template <typename T, int R, int INNER>
 cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                        int64_t S, int k, bool vec, cudaStream_t st) {
+                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr) {
   constexpr int LR = ilog2c(R);
-  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st);
+  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st, nr);
   switch (k) {
-    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st);
-    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st); break;
-    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st); break;
-    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st); break;
+    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st, nr);
+    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st, nr); break;
+    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st, nr); break;
+    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st, nr); break;
   }
   return cudaErrorInvalidValue;
 }
@@ -228,8 +232,8 @@ int tma_mode() { static int v = env_int("TRIDIAG_TMA", 1); return v; }
 
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                       int64_t S, int k, bool vec, cudaStream_t st) {
-  if (vec && k >= ilog2c(R) && tma_mode()) {
+                       int64_t S, int k, bool vec, cudaStream_t st, int64_t nr) {
+  if (vec && nr == n && k >= ilog2c(R) && tma_mode()) {
     bool used = false;
     const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
     if (used || e != cudaSuccess) return e;
@@ -244,14 +248,16 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
   const int pm = prefetch_mode();
   const int pf = vec && (pm == 1 || pm == 2) ? 1 : 0;
-  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf);
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf,
+                                             (int)nr, c_pad);
   g_last_launches = 1;
   return cudaGetLastError();
 }
 
 template <typename T, int INNER>
 cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const void* d_, void* x_,
-                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype) {
+                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr) {
   const T* a = static_cast<const T*>(a_);
   const T* b = static_cast<const T*>(b_);
   const T* c = static_cast<const T*>(c_);
@@ -260,32 +266,32 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
   const Plan p = plan_for(dtype, n, S);
   const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
   auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
-  const bool vec = al(a) && al(b) && al(c) && al(d) && al(x);
+  const bool vec = nr == n && al(a) && al(b) && al(c) && al(d) && al(x);
   if (!p.cta) {
     switch (p.R) {
-      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
       case 16:
-        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
         break;
     }
     return cudaErrorInvalidValue;
   }
   if constexpr (sizeof(T) == 4) {
     switch (p.W) {
-      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
     }
   } else {
     switch (p.W) {
-      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st);
-      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st);
+      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
     }
   }
   return cudaErrorInvalidValue;
@@ -304,17 +310,18 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
   if (S != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
   if (algo < TRIDIAG_CR || algo > TRIDIAG_CR_RD) return TRIDIAG_ERR_ALGO;
-  if (n < 2 || !is_pow2(n)) return TRIDIAG_ERR_N;
-  if (n > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
+  if (n < 1) return TRIDIAG_ERR_N;
+  const int64_t np = pad_n(n);
+  if (np > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
   if (S < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
   int64_t m;
   if (algo == TRIDIAG_CR) m = 2;
-  else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD) m = n;
-  else m = switch_level == 0 ? tridiag_auto_switch_level(n, dtype, algo) : switch_level;
+  else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD) m = np;
+  else m = switch_level == 0 ? tridiag_auto_switch_level(np, dtype, algo) : switch_level;
   if (!is_hybrid(algo) && switch_level != 0) return TRIDIAG_ERR_SWITCH_LEVEL;
   if (is_hybrid(algo)) {
-    if (switch_level < 0 || m < 2 || !is_pow2(m) || m > n ||
-        m > tridiag_max_switch_level(dtype, algo, n))
+    if (switch_level < 0 || m < 2 || !is_pow2(m) || m > np ||
+        m > tridiag_max_switch_level(dtype, algo, np))
       return TRIDIAG_ERR_SWITCH_LEVEL;
   }
   const size_t bytes = (size_t)n * (size_t)S * elem_size(dtype);
@@ -326,18 +333,19 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
   return TRIDIAG_OK;
 }
 
-int solve_device(const void* a, const void* b, const void* c, const void* d, void* x, int64_t n,
+int solve_device(const void* a, const void* b, const void* c, const void* d, void* x, int64_t nr,
                  int64_t S, int dtype, int algo, int64_t m, cudaStream_t st) {
   if (S == 0) return TRIDIAG_OK;
+  const int64_t n = pad_n(nr);
   const int k = ilog2_64(n / m);
   const int inner = (algo == TRIDIAG_RD || algo == TRIDIAG_CR_RD) ? tdg::kRD : tdg::kPCR;
   cudaError_t e;
   if (dtype == TRIDIAG_F32)
-    e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype)
-                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype);
+    e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr)
+                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr);
   else
-    e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype)
-                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype);
+    e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr)
+                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr);
   return e == cudaSuccess ? TRIDIAG_OK : (int)e;
 }
 
@@ -353,7 +361,7 @@ const char* tridiag_status_string(int status) {
   switch (status) {
     case TRIDIAG_OK: return "ok";
     case TRIDIAG_ERR_NULL: return "null pointer argument";
-    case TRIDIAG_ERR_N: return "n must be a power of two >= 2";
+    case TRIDIAG_ERR_N: return "n must be >= 1";
     case TRIDIAG_ERR_N_TOO_LARGE: return "n exceeds tridiag_max_n(dtype, algo)";
     case TRIDIAG_ERR_NUM_SYSTEMS: return "num_systems must be >= 0";
     case TRIDIAG_ERR_DTYPE: return "invalid dtype";
@@ -380,14 +388,14 @@ int64_t tridiag_max_n(int dtype, int algo) {
 
 int64_t tridiag_max_switch_level(int dtype, int algo, int64_t n) {
   if (!is_hybrid(algo) || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
-  if (n < 2 || !is_pow2(n) || n > max_n_cr(dtype)) return 0;
-  return std::min<int64_t>(n, max_inner_m(dtype));
+  if (n < 1 || pad_n(n) > max_n_cr(dtype)) return 0;
+  return std::min<int64_t>(pad_n(n), max_inner_m(dtype));
 }
 
 int tridiag_auto_switch_level(int64_t n, int dtype, int algo) {
   if (!is_hybrid(algo) || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
-  if (n < 2 || !is_pow2(n) || n > max_n_cr(dtype)) return 0;
-  return auto_m(n, dtype, algo);
+  if (n < 1 || pad_n(n) > max_n_cr(dtype)) return 0;
+  return auto_m(pad_n(n), dtype, algo);
 }
 
 int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d, void* x,

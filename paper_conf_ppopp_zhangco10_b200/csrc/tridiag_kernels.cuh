@@ -51,7 +51,8 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
 template <typename T, int R, int INNER, int KB>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf) {
+                const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
+                int n_real, T c_pad) {
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -70,13 +71,20 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     }
     const long long sys = s0 + sub;
     const bool valid = sys < S;
-    const size_t off = (size_t)sys * (size_t)n + (size_t)ls * R;
+    const bool ragged = n_real != n;  // uniform
+    const size_t sbase = (size_t)sys * (size_t)n_real;
+    const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
-    if (valid) {
+    if (valid && !ragged) {
       load_block<T, R, true>(a + off, ra, vec);
       load_block<T, R, true>(b + off, rb, vec);
       load_block<T, R, true>(c + off, rc, vec);
       load_block<T, R, false>(d + off, rd, vec);
+    } else if (valid) {
+      load_ragged<T, R>(a + sbase, ls * R, n_real, ra, T(0), T(0), false);
+      load_ragged<T, R>(b + sbase, ls * R, n_real, rb, T(1), T(0), false);
+      load_ragged<T, R>(c + sbase, ls * R, n_real, rc, c_pad, c_pad, true);
+      load_ragged<T, R>(d + sbase, ls * R, n_real, rd, T(0), T(0), false);
     } else {
 #pragma unroll
       for (int i = 0; i < R; ++i) { ra[i] = T(0); rb[i] = T(1); rc[i] = T(0); rd[i] = T(0); }
@@ -85,7 +93,10 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
-    if (valid) store_block<T, R>(x + off, rd, vec);
+    if (valid) {
+      if (!ragged) store_block<T, R>(x + off, rd, vec);
+      else store_ragged<T, R>(x + sbase, ls * R, n_real, rd);
+    }
   }
 }
 
@@ -255,7 +266,8 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
 template <typename T, int R, int W, int INNER, bool SMEM>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-               const T* d, T* x, int n, long long S, int k, int vec, int pf) {
+               const T* d, T* x, int n, long long S, int k, int vec, int pf, int n_real,
+               T c_pad) {
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;
@@ -275,12 +287,21 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       prefetch_l2(base + (size_t)(sys + gridDim.x) * n + (size_t)warp * 32 * R,
                   (uint32_t)(32 * R * sizeof(T)));
     }
-    const size_t off = (size_t)sys * (size_t)n + (size_t)ls * R;
+    const bool ragged = n_real != n;
+    const size_t sbase = (size_t)sys * (size_t)n_real;
+    const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
-    load_block<T, R, true>(a + off, ra, vec);
-    load_block<T, R, true>(b + off, rb, vec);
-    load_block<T, R, true>(c + off, rc, vec);
-    load_block<T, R, false>(d + off, rd, vec);
+    if (!ragged) {
+      load_block<T, R, true>(a + off, ra, vec);
+      load_block<T, R, true>(b + off, rb, vec);
+      load_block<T, R, true>(c + off, rc, vec);
+      load_block<T, R, false>(d + off, rd, vec);
+    } else {
+      load_ragged<T, R>(a + sbase, ls * R, n_real, ra, T(0), T(0), false);
+      load_ragged<T, R>(b + sbase, ls * R, n_real, rb, T(1), T(0), false);
+      load_ragged<T, R>(c + sbase, ls * R, n_real, rc, c_pad, c_pad, true);
+      load_ragged<T, R>(d + sbase, ls * R, n_real, rd, T(0), T(0), false);
+    }
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
 
@@ -316,7 +337,8 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       xprev = ls > 0 ? X[ls * q - 1] : T(0);
     }
     inlane_backward<T, R>(ra, rb, rc, rd, kin, xprev);
-    store_block<T, R>(x + off, rd, vec);
+    if (!ragged) store_block<T, R>(x + off, rd, vec);
+    else store_ragged<T, R>(x + sbase, ls * R, n_real, rd);
     __syncthreads();  // shared memory is reused by the next system
   }
 }

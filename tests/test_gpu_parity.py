@@ -203,6 +203,41 @@ def test_rd_on_dd_reports_instability_not_errors():
         assert (e > 1e-4).any()
 
 
+# --------------------------------------------------------------------------- ragged n (NEXT f2)
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_ragged_n(dtype):
+    """n not a power of two: solved as the next power of two with decoupled
+    padding equations (c_pad = 0; RD c_pad = 1); only the n real elements are
+    read or written.  Gate against Thomas (any n)."""
+    for n in [1, 3, 5, 17, 33, 100, 257, 511, 513, 1000, 3000]:
+        for algo, fam in [("cr", "dd"), ("cr_pcr", "dd"), ("pcr", "dd"), ("rd", "poi"), ("cr_rd", "poi")]:
+            if n > td.max_n(dtype, algo) or (algo == "rd" and dtype == torch.float32 and n > 32):
+                continue
+            a, b, c, d = gen(fam, 45, n, dtype, seed=n)
+            x = gpu_solve(a, b, c, d, algo)
+            e = err_vs_oracle(a, b, c, d, x)
+            assert e.max() <= TOL[dtype], (algo, n, e.max())
+        # corners are still ignored; neighbours of the batch untouched
+        ap, bp, cp, dp = gen("dd", 45, n, dtype, seed=n, poison_corners=True)
+        a, b, c, d = gen("dd", 45, n, dtype, seed=n)
+        assert torch.equal(gpu_solve(a, b, c, d, "cr_pcr"), gpu_solve(ap, bp, cp, dp, "cr_pcr"))
+        guard = torch.full((47 * n,), 7.0, dtype=dtype, device="cuda")
+        xv = guard[n:46 * n].view(45, n)
+        td.solve_batched(a, b, c, d, x=xv, algo="cr_pcr")
+        torch.cuda.synchronize()
+        assert torch.all(guard[:n] == 7.0) and torch.all(guard[46 * n:] == 7.0)
+
+
+def test_ragged_closed_form():
+    for n in [3, 7, 100, 500]:
+        for dtype in (torch.float32, torch.float64):
+            a, b, c, d = gen("poi1", 8, n, dtype)
+            i = np.arange(n, dtype=np.float64)
+            ref = (i + 1.0) * (n - i) / 2.0
+            x = host(gpu_solve(a, b, c, d, "cr"))[0].astype(np.float64)
+            assert np.max(np.abs(x - ref)) / ref.max() <= 8 * float(torch.finfo(dtype).eps), n
+
+
 # --------------------------------------------------------------------------- edge cases
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
 def test_corner_poisoning_is_ignored(dtype):
