@@ -47,10 +47,14 @@ int64_t max_n_cr(int dtype) { return dtype == TRIDIAG_F64 ? 4096 : 8192; }
 // the best time (8), because RD's error grows with m on dominant input
 // (R24).
 int lanes_per_system(int dtype, int64_t n);
+bool cta_plan(int dtype, int64_t n);
 int auto_m(int64_t n, int dtype, int algo) {
   if (!is_hybrid(algo)) return 0;
   const int64_t P = lanes_per_system(dtype, n);
-  int64_t m = algo == TRIDIAG_CR_PCR ? std::min<int64_t>(P, 32) : std::min<int64_t>(P, 8);
+  // CTA plans (n > 32 R): m = 32 is >= 5% faster than m = 8 for CR+RD too
+  // (fewer in-warp lane-level levels), so it is the tuned choice there.
+  int64_t m = (algo == TRIDIAG_CR_PCR || cta_plan(dtype, n)) ? std::min<int64_t>(P, 32)
+                                                             : std::min<int64_t>(P, 8);
   if (m < 2) m = 2;
   if (m > n) m = n;
   return (int)m;
@@ -97,6 +101,8 @@ Plan plan_for(int dtype, int64_t n, int64_t S = -1) {
 
 // Lanes per system of the HBM-scale plan: the largest m the hybrids keep on
 // the register path (the small-batch plan has at least as many lanes).
+bool cta_plan(int dtype, int64_t n) { return plan_for(dtype, n).cta; }
+
 int lanes_per_system(int dtype, int64_t n) {
   const Plan p = plan_for(dtype, n);
   return p.cta ? 32 : (int)(n / p.R);
