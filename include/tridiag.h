@@ -51,7 +51,8 @@ enum {
     TRIDIAG_ERR_ALGO = -6,         /* algo not a tridiag_algo                        */
     TRIDIAG_ERR_SWITCH_LEVEL = -7, /* invalid switch_level for this algo / n / dtype */
     TRIDIAG_ERR_OVERLAP = -8,      /* x overlaps an input other than exactly x == d  */
-    TRIDIAG_ERR_WORKSPACE = -9     /* host entry point: workspace too small / NULL   */
+    TRIDIAG_ERR_WORKSPACE = -9,    /* host entry point: workspace too small / NULL   */
+    TRIDIAG_ERR_STRIDE = -10       /* strided entry point: invalid strides           */
 };
 
 /*
@@ -103,6 +104,26 @@ enum {
 int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d,
                           void* x, int64_t n, int64_t num_systems, int dtype, int algo,
                           int switch_level, tridiag_stream_t stream);
+
+/*
+ * tridiag_solve_batched_strided -- the same solve for strided layouts
+ * (SURVEY.md 8(f) NEXT f1): element i of system s of every array is at
+ * ptr[s * sys_stride + i * elem_stride] (strides in elements, >= 1, one of
+ * them 1, the mapping one-to-one: sys_stride >= elem_stride * n or
+ * elem_stride >= sys_stride * num_systems).  (1, n) is the contiguous layout
+ * of tridiag_solve_batched; (1, pitch) a pitched row sweep; (es, 1) with
+ * es >= num_systems is the ADI column sweep of a row-major grid ("the most
+ * common application", ADI): e.g. the columns of an
+ * NY x NX grid are NX systems of n = NY with elem_stride = NX, sys_stride = 1.
+ * Interleaved layouts are staged through shared memory in tiles of 8
+ * consecutive systems (coalesced 32-byte rows); other non-contiguous layouts
+ * use scalar loads.  x must use the same strides; x == d is allowed.
+ * Errors as tridiag_solve_batched plus TRIDIAG_ERR_STRIDE.
+ */
+int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, const void* d,
+                                  void* x, int64_t n, int64_t num_systems, int64_t elem_stride,
+                                  int64_t sys_stride, int dtype, int algo, int switch_level,
+                                  tridiag_stream_t stream);
 
 /*
  * tridiag_solve_batched_host -- the same solve for HOST arrays (the paper's

@@ -12,7 +12,7 @@ CSRC = os.path.join(PKG, "csrc")
 INCLUDE = os.path.join(ROOT, "include")
 LIB = os.path.join(PKG, "libtridiag.so")
 SOURCES = ["tridiag_api.cu"]
-DEPS = SOURCES + ["tridiag_device.cuh", "tridiag_kernels.cuh", "tridiag_tma.cuh"]
+DEPS = SOURCES + ["tridiag_device.cuh", "tridiag_kernels.cuh", "tridiag_tma.cuh", "tridiag_ileave.cuh"]
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",

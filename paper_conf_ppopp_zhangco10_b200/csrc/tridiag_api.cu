@@ -12,6 +12,7 @@
 #include <tuple>
 
 #include "tridiag.h"
+#include "tridiag_ileave.cuh"
 #include "tridiag_tma.cuh"
 
 #include <cudaTypedefs.h>
@@ -136,9 +137,36 @@ int occupancy(int dev, K kernel, int threads, size_t smem) {
   return nb;
 }
 
+struct Layout {
+  int64_t es, ss;  // element stride, system stride (elements)
+};
+
+template <typename T, int R, int INNER, int KB>
+cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                            int64_t S, int k, cudaStream_t st, int64_t n_real, Layout L) {
+  const int P = (int)(n / R);
+  const int G = std::max(8, 32 / P);
+  const int threads = G * P;
+  const size_t smem = (size_t)4 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
+  if (smem > 227 * 1024) return cudaErrorInvalidValue;
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = tdg::tdg_ileave_kernel<T, R, INNER, KB>;
+  const int occ = occupancy(dev, kern, threads, smem);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t tiles = (S + G - 1) / G;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)device_sms(dev) * occ));
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, ilog2c(P), G,
+                                              (int)n_real, c_pad, (long long)L.es);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
 template <typename T, int R, int INNER, int KB>
 cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                          int64_t S, int k, bool vec, cudaStream_t st, int64_t n_real) {
+                          int64_t S, int k, bool vec, cudaStream_t st, int64_t n_real, Layout L) {
+  if (L.ss == 1 && L.es != 1) return launch_ileave_k<T, R, INNER, KB>(a, b, c, d, x, n, S, k, st, n_real, L);
   const int P = (int)(n / R);
   const int log2P = ilog2c(P);
   const int G = 32 / P;
@@ -155,7 +183,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
-                                           vec ? 1 : 0, pf, (int)n_real, c_pad);
+                                           vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
+                                           (long long)L.ss);
   g_last_launches = 1;
   return cudaGetLastError();
 }
@@ -164,14 +193,14 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
 // blocked-inner kernel compiled for that k.
 template <typename T, int R, int INNER>
 cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr) {
+                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
   constexpr int LR = ilog2c(R);
-  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st, nr);
+  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st, nr, L);
   switch (k) {
-    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st, nr);
-    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st, nr); break;
-    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st, nr); break;
-    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st, nr); break;
+    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
+    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
+    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
   }
   return cudaErrorInvalidValue;
 }
@@ -238,8 +267,8 @@ int tma_mode() { static int v = env_int("TRIDIAG_TMA", 1); return v; }
 
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                       int64_t S, int k, bool vec, cudaStream_t st, int64_t nr) {
-  if (vec && nr == n && k >= ilog2c(R) && tma_mode()) {
+                       int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
+  if (vec && nr == n && L.es == 1 && L.ss == n && k >= ilog2c(R) && tma_mode()) {
     bool used = false;
     const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
     if (used || e != cudaSuccess) return e;
@@ -256,14 +285,15 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   const int pf = vec && (pm == 1 || pm == 2) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf,
-                                             (int)nr, c_pad);
+                                             (int)nr, c_pad, (long long)L.es, (long long)L.ss);
   g_last_launches = 1;
   return cudaGetLastError();
 }
 
 template <typename T, int INNER>
 cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const void* d_, void* x_,
-                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr) {
+                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr,
+                       Layout L) {
   const T* a = static_cast<const T*>(a_);
   const T* b = static_cast<const T*>(b_);
   const T* c = static_cast<const T*>(c_);
@@ -272,32 +302,33 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
   const Plan p = plan_for(dtype, n, S);
   const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
   auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
-  const bool vec = nr == n && al(a) && al(b) && al(c) && al(d) && al(x);
+  const bool vec = nr == n && L.es == 1 && ((uint64_t)L.ss * sizeof(T)) % tile == 0 && al(a) &&
+                   al(b) && al(c) && al(d) && al(x);
   if (!p.cta) {
     switch (p.R) {
-      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
       case 16:
-        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
         break;
     }
     return cudaErrorInvalidValue;
   }
   if constexpr (sizeof(T) == 4) {
     switch (p.W) {
-      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
     }
   } else {
     switch (p.W) {
-      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
-      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr);
+      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
     }
   }
   return cudaErrorInvalidValue;
@@ -311,7 +342,8 @@ bool overlaps(const void* p, const void* q, size_t bytes) {
 // Host-side argument validation (integer only; nothing is enqueued on error).
 // On success *m_out is the resolved intermediate size m (n for PCR/RD, 2 for CR).
 int validate(const void* a, const void* b, const void* c, const void* d, const void* x,
-             int64_t n, int64_t S, int dtype, int algo, int switch_level, int64_t* m_out) {
+             int64_t n, int64_t S, int dtype, int algo, int switch_level, int64_t* m_out,
+             int64_t es, int64_t ss) {
   // NULL pointers are legal only for an empty batch (nothing is accessed).
   if (S != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
@@ -330,7 +362,11 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
         m > tridiag_max_switch_level(dtype, algo, np))
       return TRIDIAG_ERR_SWITCH_LEVEL;
   }
-  const size_t bytes = (size_t)n * (size_t)S * elem_size(dtype);
+  // strides: element (s, i) at s*ss + i*es must be one-to-one (one index nests the other)
+  if (es < 1 || ss < 1) return TRIDIAG_ERR_STRIDE;
+  if (S > 1 && n > 1 && !(ss >= es * n || es >= ss * S)) return TRIDIAG_ERR_STRIDE;
+  if (n > 1 && S > 1 && es > 1 && ss > 1) return TRIDIAG_ERR_STRIDE;  // one stride must be 1
+  const size_t bytes = S > 0 ? (size_t)((S - 1) * ss + (n - 1) * es + 1) * elem_size(dtype) : 0;
   if (bytes > 0) {
     if (overlaps(x, a, bytes) || overlaps(x, b, bytes) || overlaps(x, c, bytes)) return TRIDIAG_ERR_OVERLAP;
     if (x != d && overlaps(x, d, bytes)) return TRIDIAG_ERR_OVERLAP;
@@ -340,18 +376,18 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
 }
 
 int solve_device(const void* a, const void* b, const void* c, const void* d, void* x, int64_t nr,
-                 int64_t S, int dtype, int algo, int64_t m, cudaStream_t st) {
+                 int64_t S, int dtype, int algo, int64_t m, cudaStream_t st, Layout L) {
   if (S == 0) return TRIDIAG_OK;
   const int64_t n = pad_n(nr);
   const int k = ilog2_64(n / m);
   const int inner = (algo == TRIDIAG_RD || algo == TRIDIAG_CR_RD) ? tdg::kRD : tdg::kPCR;
   cudaError_t e;
   if (dtype == TRIDIAG_F32)
-    e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr)
-                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr);
+    e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
+                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
   else
-    e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr)
-                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr);
+    e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
+                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
   return e == cudaSuccess ? TRIDIAG_OK : (int)e;
 }
 
@@ -375,6 +411,7 @@ const char* tridiag_status_string(int status) {
     case TRIDIAG_ERR_SWITCH_LEVEL: return "invalid switch_level for this algo/n/dtype";
     case TRIDIAG_ERR_OVERLAP: return "x overlaps an input (only x == d is allowed)";
     case TRIDIAG_ERR_WORKSPACE: return "workspace missing or too small";
+    case TRIDIAG_ERR_STRIDE: return "invalid strides (need >= 1, one of them 1, non-overlapping)";
   }
   if (status > 0) return cudaGetErrorString((cudaError_t)status);
   return "unknown status";
@@ -404,15 +441,24 @@ int tridiag_auto_switch_level(int64_t n, int dtype, int algo) {
   return auto_m(pad_n(n), dtype, algo);
 }
 
+int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, const void* d,
+                                  void* x, int64_t n, int64_t num_systems, int64_t elem_stride,
+                                  int64_t sys_stride, int dtype, int algo, int switch_level,
+                                  tridiag_stream_t stream) {
+  g_last_launches = 0;
+  int64_t m = 0;
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m,
+                         elem_stride, sys_stride);
+  if (v != TRIDIAG_OK) return v;
+  return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, m,
+                      reinterpret_cast<cudaStream_t>(stream), Layout{elem_stride, sys_stride});
+}
+
 int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d, void* x,
                           int64_t n, int64_t num_systems, int dtype, int algo, int switch_level,
                           tridiag_stream_t stream) {
-  g_last_launches = 0;
-  int64_t m = 0;
-  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m);
-  if (v != TRIDIAG_OK) return v;
-  return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, m,
-                      reinterpret_cast<cudaStream_t>(stream));
+  return tridiag_solve_batched_strided(a, b, c, d, x, n, num_systems, 1, n, dtype, algo,
+                                       switch_level, stream);
 }
 
 size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems) {
@@ -427,7 +473,7 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
                                int64_t chunk_systems) {
   g_last_launches = 0;
   int64_t m = 0;
-  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m);
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, 1, n);
   if (v != TRIDIAG_OK) return v;
   if (num_systems == 0) return TRIDIAG_OK;
   if (chunk_systems < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
@@ -463,7 +509,7 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
     if (rc != TRIDIAG_OK) break;
     // x overwrites the chunk's d in place on the device.
     rc = solve_device(buf, buf + arr, buf + 2 * arr, buf + 3 * arr, buf + 3 * arr, n, cnt, dtype,
-                      algo, m, s);
+                      algo, m, s, Layout{1, n});
     launches += g_last_launches;
     if (rc != TRIDIAG_OK) break;
     cudaError_t e = cudaMemcpyAsync(hx + off, buf + 3 * arr, bytes, cudaMemcpyDeviceToHost, s);

@@ -52,7 +52,7 @@ template <typename T, int R, int INNER, int KB>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
-                int n_real, T c_pad) {
+                int n_real, T c_pad, long long es, long long ss) {
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -71,8 +71,9 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     }
     const long long sys = s0 + sub;
     const bool valid = sys < S;
-    const bool ragged = n_real != n;  // uniform
-    const size_t sbase = (size_t)sys * (size_t)n_real;
+    // general (scalar, strided and/or padded) path unless contiguous power of two
+    const bool ragged = n_real != n || es != 1;  // uniform
+    const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
     if (valid && !ragged) {
@@ -81,10 +82,10 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
       load_block<T, R, true>(c + off, rc, vec);
       load_block<T, R, false>(d + off, rd, vec);
     } else if (valid) {
-      load_ragged<T, R>(a + sbase, ls * R, n_real, ra, T(0), T(0), false);
-      load_ragged<T, R>(b + sbase, ls * R, n_real, rb, T(1), T(0), false);
-      load_ragged<T, R>(c + sbase, ls * R, n_real, rc, c_pad, c_pad, true);
-      load_ragged<T, R>(d + sbase, ls * R, n_real, rd, T(0), T(0), false);
+      load_ragged<T, R>(a + sbase, es, ls * R, n_real, ra, T(0), T(0), false);
+      load_ragged<T, R>(b + sbase, es, ls * R, n_real, rb, T(1), T(0), false);
+      load_ragged<T, R>(c + sbase, es, ls * R, n_real, rc, c_pad, c_pad, true);
+      load_ragged<T, R>(d + sbase, es, ls * R, n_real, rd, T(0), T(0), false);
     } else {
 #pragma unroll
       for (int i = 0; i < R; ++i) { ra[i] = T(0); rb[i] = T(1); rc[i] = T(0); rd[i] = T(0); }
@@ -95,7 +96,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
     if (valid) {
       if (!ragged) store_block<T, R>(x + off, rd, vec);
-      else store_ragged<T, R>(x + sbase, ls * R, n_real, rd);
+      else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
     }
   }
 }
@@ -267,7 +268,7 @@ template <typename T, int R, int W, int INNER, bool SMEM>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                const T* d, T* x, int n, long long S, int k, int vec, int pf, int n_real,
-               T c_pad) {
+               T c_pad, long long es, long long ss) {
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;
@@ -287,8 +288,8 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       prefetch_l2(base + (size_t)(sys + gridDim.x) * n + (size_t)warp * 32 * R,
                   (uint32_t)(32 * R * sizeof(T)));
     }
-    const bool ragged = n_real != n;
-    const size_t sbase = (size_t)sys * (size_t)n_real;
+    const bool ragged = n_real != n || es != 1;
+    const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
     if (!ragged) {
@@ -297,10 +298,10 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       load_block<T, R, true>(c + off, rc, vec);
       load_block<T, R, false>(d + off, rd, vec);
     } else {
-      load_ragged<T, R>(a + sbase, ls * R, n_real, ra, T(0), T(0), false);
-      load_ragged<T, R>(b + sbase, ls * R, n_real, rb, T(1), T(0), false);
-      load_ragged<T, R>(c + sbase, ls * R, n_real, rc, c_pad, c_pad, true);
-      load_ragged<T, R>(d + sbase, ls * R, n_real, rd, T(0), T(0), false);
+      load_ragged<T, R>(a + sbase, es, ls * R, n_real, ra, T(0), T(0), false);
+      load_ragged<T, R>(b + sbase, es, ls * R, n_real, rb, T(1), T(0), false);
+      load_ragged<T, R>(c + sbase, es, ls * R, n_real, rc, c_pad, c_pad, true);
+      load_ragged<T, R>(d + sbase, es, ls * R, n_real, rd, T(0), T(0), false);
     }
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
@@ -338,7 +339,7 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
     }
     inlane_backward<T, R>(ra, rb, rc, rd, kin, xprev);
     if (!ragged) store_block<T, R>(x + off, rd, vec);
-    else store_ragged<T, R>(x + sbase, ls * R, n_real, rd);
+    else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
     __syncthreads();  // shared memory is reused by the next system
   }
 }

@@ -49,6 +49,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         P, I64, I = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int
         L.tridiag_solve_batched.argtypes = [P, P, P, P, P, I64, I64, I, I, I, P]
         L.tridiag_solve_batched.restype = I
+        L.tridiag_solve_batched_strided.argtypes = [P, P, P, P, P, I64, I64, I64, I64, I, I, I, P]
+        L.tridiag_solve_batched_strided.restype = I
         L.tridiag_solve_batched_host.argtypes = [P, P, P, P, P, I64, I64, I, I, I, P,
                                                  ctypes.c_size_t, I64]
         L.tridiag_solve_batched_host.restype = I
@@ -123,14 +125,27 @@ def solve_batched_raw(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, n, num_systems, dtype, 
                                        int(switch_level), stream))
 
 
-def _check_tensors(ts, device_kind):
+def solve_batched_strided_raw(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, n, num_systems, elem_stride,
+                              sys_stride, dtype, algo, switch_level=0, stream=0) -> int:
+    """Direct C-ABI call of tridiag_solve_batched_strided; returns the status."""
+    L = load()
+    return int(L.tridiag_solve_batched_strided(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, int(n),
+                                               int(num_systems), int(elem_stride),
+                                               int(sys_stride), _dtype_code(dtype),
+                                               _algo_code(algo), int(switch_level), stream))
+
+
+def _check_tensors(ts, device_kind, same_strides=False):
     t0 = ts[0]
     if t0.dim() != 2:
         raise ValueError("tensors must be (num_systems, n)")
     for t in ts:
         if t.shape != t0.shape or t.dtype != t0.dtype:
             raise ValueError("a, b, c, d, x must share shape and dtype")
-        if not t.is_contiguous():
+        if same_strides:
+            if t.stride() != t0.stride():
+                raise ValueError("a, b, c, d, x must share strides")
+        elif not t.is_contiguous():
             raise ValueError("tensors must be contiguous")
         if device_kind == "cuda" and (not t.is_cuda or t.device != t0.device):
             raise ValueError("tensors must be on the same CUDA device")
@@ -143,22 +158,31 @@ def _check_tensors(ts, device_kind):
 def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None):
     """Solve the (S, n) batch a_i x_{i-1} + b_i x_i + c_i x_{i+1} = d_i on the GPU.
 
-    a, b, c, d: contiguous CUDA tensors (float32/float64) of shape (S, n).
-    x: output tensor (may be d itself for in-place); allocated if None.
+    a, b, c, d: CUDA tensors (float32/float64) of shape (S, n) -- row s is
+    system s -- with identical strides: contiguous, pitched rows, or
+    transposed views such as ``grid.T`` for the column sweep of ADI
+    (tridiag_solve_batched_strided).
+    x: output tensor with the same strides (may be d itself); allocated if None.
     algo: 'cr' | 'pcr' | 'rd' | 'cr_pcr' | 'cr_rd'.
     switch_level: intermediate size m of the hybrids (0 = tuned table).
     Enqueued asynchronously on ``stream`` (default: torch's current stream).
     """
     if x is None:
-        x = torch.empty_like(d)
-    _check_tensors([a, b, c, d, x], "cuda")
+        x = torch.empty_strided(d.shape, d.stride(), dtype=d.dtype, device=d.device)
+    _check_tensors([a, b, c, d, x], "cuda", same_strides=True)
     S, n = d.shape
+    ss, es = d.stride()
     if stream is None:
         stream = torch.cuda.current_stream(d.device)
     with torch.cuda.device(d.device):
-        st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
-                               x.data_ptr(), n, S, d.dtype, algo, switch_level,
-                               stream.cuda_stream)
+        if es == 1 and (ss == n or S <= 1):
+            st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                   x.data_ptr(), n, S, d.dtype, algo, switch_level,
+                                   stream.cuda_stream)
+        else:
+            st = solve_batched_strided_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                           x.data_ptr(), n, S, es, max(ss, 1), d.dtype, algo,
+                                           switch_level, stream.cuda_stream)
     check(st)
     return x
 

@@ -129,3 +129,22 @@ def test_host_workspace_size():
     # workspace too small -> -9 before any CUDA call
     st = L.tridiag_solve_batched_host(A, B, C, D, X, 512, 4, F32, CR, 0, 0x1000, 16, 2)
     assert st == -9
+
+
+def strided(n=512, S=4, es=1, ss=512, **kw):
+    args = dict(a=A, b=B, c=C, d=D, x=X, dtype=F32, algo=CR, m=0)
+    args.update(kw)
+    return td.solve_batched_strided_raw(args["a"], args["b"], args["c"], args["d"], args["x"], n, S,
+                                        es, ss, args["dtype"], args["algo"], args["m"], None)
+
+
+def test_stride_validation():
+    assert strided(es=0, S=0) == -10
+    assert strided(ss=0, S=0) == -10
+    assert strided(es=2, ss=2000, S=4) == -10      # neither stride is 1
+    assert strided(es=1, ss=100, S=4) == -10       # rows overlap (ss < n)
+    assert strided(es=3, ss=1, S=4, n=8) == -10    # columns overlap (es < S)
+    assert strided(es=1, ss=512, S=0) == 0         # contiguous
+    assert strided(es=1, ss=600, S=0) == 0         # pitched rows
+    assert strided(es=8, ss=1, S=0, n=8) == 0      # interleaved
+    assert td.status_string(-10).startswith("invalid strides")

@@ -238,6 +238,54 @@ def test_ragged_closed_form():
             assert np.max(np.abs(x - ref)) / ref.max() <= 8 * float(torch.finfo(dtype).eps), n
 
 
+# --------------------------------------------------------------------------- strided (NEXT f1)
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_adi_column_sweep_interleaved(dtype):
+    """Columns of a row-major NY x NX grid (elem stride NX, system stride 1):
+    the ADI column sweep.  Same results as solving the
+    contiguous copies, bitwise, and within the gate vs the oracle."""
+    for NY, NX in [(64, 40), (512, 1000), (256, 9), (100, 37), (2048, 50)]:
+        grids = inputs.generate("dd", NX, NY, dtype, seed=NY)  # (NX systems, NY eqs)
+        # lay them out as columns of (NY, NX) row-major grids
+        G = [g.t().contiguous() for g in grids]                  # (NY, NX), column j = system j
+        views = [g.t() for g in G]                               # (NX, NY) strides (1, NX)
+        assert views[0].stride() == (1, NX)
+        for algo in ["cr", "cr_pcr", "pcr"]:
+            if NY > td.max_n(dtype, algo):
+                continue
+            x = gpu_solve(*views, algo)
+            assert x.stride() == (1, NX)
+            ref = gpu_solve(*[g.contiguous() for g in grids], algo)
+            assert torch.equal(x.contiguous(), ref), (NY, NX, algo)
+            e = err_vs_oracle(*grids, x.contiguous())
+            assert e.max() <= TOL[dtype], (NY, NX, algo, e.max())
+        # in place into the grid itself
+        td.solve_batched(*views, x=views[3], algo="cr_pcr")
+        torch.cuda.synchronize()
+        assert torch.equal(views[3].contiguous(), gpu_solve(*[g.contiguous() for g in grids], "cr_pcr"))
+
+
+def test_pitched_rows_and_rd_interleaved():
+    for dtype in (torch.float32, torch.float64):
+        S, n, pitch = 300, 512, 520
+        base = [torch.zeros(S, pitch, dtype=dtype, device="cuda") for _ in range(5)]
+        a, b, c, d = gen("dd", S, n, dtype)
+        views = [t[:, :n] for t in base]
+        for v, src in zip(views[:4], (a, b, c, d)):
+            v.copy_(src)
+        td.solve_batched(*views[:4], x=views[4], algo="cr_pcr")
+        torch.cuda.synchronize()
+        assert torch.equal(views[4], gpu_solve(a, b, c, d, "cr_pcr"))
+        assert torch.all(base[4][:, n:] == 0)
+        # RD family on an interleaved POI layout
+        p = gen("poi", 77, 128, dtype, seed=5)
+        cols = [t.t().contiguous().t() for t in p]
+        for algo in ("rd", "cr_rd"):
+            if dtype == torch.float32 and algo == "rd":
+                continue
+            assert torch.equal(gpu_solve(*cols, algo).contiguous(), gpu_solve(*p, algo)), algo
+
+
 # --------------------------------------------------------------------------- edge cases
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
 def test_corner_poisoning_is_ignored(dtype):
