@@ -245,7 +245,7 @@ def test_adi_column_sweep_interleaved(dtype):
     the ADI column sweep.  Same results as solving the
     contiguous copies, bitwise, and within the gate vs the oracle."""
     for NY, NX in [(64, 40), (512, 1000), (256, 9), (100, 37), (2048, 50)]:
-        grids = inputs.generate("dd", NX, NY, dtype, seed=NY)  # (NX systems, NY eqs)
+        grids = gen("dd", NX, NY, dtype, seed=NY)  # (NX systems, NY eqs)
         # lay them out as columns of (NY, NX) row-major grids
         G = [g.t().contiguous() for g in grids]                  # (NY, NX), column j = system j
         views = [g.t() for g in G]                               # (NX, NY) strides (1, NX)

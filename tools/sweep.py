@@ -199,9 +199,37 @@ def c4(args):
               "frac_of_peak": per / med / 1e9 / PEAK})
 
 
+def adi(args):
+    """ADI-style 2D sweeps on NY x NX row-major grids: the row sweep solves NY
+    contiguous systems of n = NX, the column sweep NX interleaved systems of
+    n = NY (element stride NX).  Both directions, CR+PCR, DD."""
+    for dts in ("f32", "f64"):
+        dt = torch.float32 if dts == "f32" else torch.float64
+        T = 4 if dts == "f32" else 8
+        for NY, NX in [(512, 131072), (256, 262144), (4096, 4096), (1024, 65536)]:
+            if NY > td.max_n(dt, "cr_pcr") or NX > 262144:
+                continue
+            nsets = max(1, math.ceil(4 * L2_BYTES / (5 * NY * NX * T)))
+            sets = []
+            for kk in range(nsets):
+                g = inputs.generate("dd", NX, NY, dt, s0=kk * NX, device="cuda")  # columns as rows
+                cols = [t.t().contiguous().t() for t in g]                          # (NX, NY) strides (1, NX)
+                sets.append((*cols, torch.empty_like(cols[0])))
+            per = 5 * NY * NX * T
+            med, mn = time_point(sets, "cr_pcr", 0, steps=args.steps)
+            emit({"config": "adi-column", "dtype": dts, "grid": [NY, NX], "n": NY, "S": NX,
+                  "ms_median": med * 1e3, "gbs": per / med / 1e9, "frac_of_peak": per / med / 1e9 / PEAK})
+            rows = [tuple(t.t() for t in st[:4]) + (st[4].t(),) for st in sets]   # (NY, NX) contiguous
+            med, mn = time_point(rows, "cr_pcr", 0, steps=args.steps)
+            emit({"config": "adi-row", "dtype": dts, "grid": [NY, NX], "n": NX, "S": NY,
+                  "ms_median": med * 1e3, "gbs": per / med / 1e9, "frac_of_peak": per / med / 1e9 / PEAK})
+            del sets, rows
+            torch.cuda.empty_cache()
+
+
 if __name__ == "__main__":
     p = argparse.ArgumentParser()
-    p.add_argument("configs", nargs="+", choices=["c2", "c3", "c4", "c5"])
+    p.add_argument("configs", nargs="+", choices=["c2", "c3", "c4", "c5", "adi"])
     p.add_argument("--steps", type=int, default=30)
     p.add_argument("--no-acc", action="store_true")
     a = p.parse_args()
