@@ -147,6 +147,10 @@ cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x
   const int P = (int)(n / R);
   const int G = std::max(8, 32 / P);
   const int threads = G * P;
+  // 16-byte vector row segments when every row segment is 16-byte aligned
+  auto a16 = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) & 15) == 0; };
+  const int vec16 = a16(a) && a16(b) && a16(c) && a16(d) && a16(x) &&
+                    ((uint64_t)L.es * sizeof(T)) % 16 == 0 ? 1 : 0;
   const size_t smem = (size_t)4 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
   if (smem > 227 * 1024) return cudaErrorInvalidValue;
   int dev = 0;
@@ -157,8 +161,8 @@ cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x
   const int64_t tiles = (S + G - 1) / G;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)device_sms(dev) * occ));
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
-  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, ilog2c(P), G,
-                                              (int)n_real, c_pad, (long long)L.es);
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, ilog2c(P),
+                                              ilog2c(G), (int)n_real, c_pad, (long long)L.es, vec16);
   g_last_launches = 1;
   return cudaGetLastError();
 }

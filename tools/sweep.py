@@ -206,8 +206,8 @@ def adi(args):
     for dts in ("f32", "f64"):
         dt = torch.float32 if dts == "f32" else torch.float64
         T = 4 if dts == "f32" else 8
-        for NY, NX in [(512, 131072), (256, 262144), (4096, 4096), (1024, 65536)]:
-            if NY > td.max_n(dt, "cr_pcr") or NX > 262144:
+        for NY, NX in [(512, 8192), (8192, 512), (4096, 4096), (2048, 2048)]:
+            if max(NY, NX) > td.max_n(dt, "cr_pcr"):
                 continue
             nsets = max(1, math.ceil(4 * L2_BYTES / (5 * NY * NX * T)))
             sets = []
