@@ -11,8 +11,10 @@ ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 INCLUDE = os.path.join(ROOT, "include")
 LIB = os.path.join(PKG, "libtridiag.so")
-SOURCES = ["tridiag_api.cu"]
-DEPS = SOURCES + ["tridiag_device.cuh", "tridiag_kernels.cuh", "tridiag_tma.cuh", "tridiag_ileave.cuh"]
+SOURCES = ["tridiag_api.cu", "inst_f32_pcr.cu", "inst_f32_rd.cu", "inst_f64_pcr.cu",
+           "inst_f64_rd.cu"]
+DEPS = SOURCES + ["tridiag_device.cuh", "tridiag_kernels.cuh", "tridiag_tma.cuh",
+                  "tridiag_ileave.cuh", "launch.cuh", "host_common.h"]
 
 NVCC_FLAGS = [
     "-gencode", "arch=compute_100a,code=sm_100a",
@@ -41,21 +43,41 @@ def _stale() -> bool:
 
 
 def build(force: bool = False, verbose: bool = False) -> str:
-    """Compile libtridiag.so if missing or older than its sources."""
+    """Compile libtridiag.so if missing or older than its sources: one nvcc per
+    translation unit (in parallel), then one link."""
     if not force and not _stale():
         return LIB
+    from concurrent.futures import ThreadPoolExecutor
+    import tempfile
+    objdir = tempfile.mkdtemp(prefix="tridiag_build_")
+    compile_flags = [f for f in NVCC_FLAGS if f != "-shared"]
+
+    def compile_one(src):
+        obj = os.path.join(objdir, os.path.splitext(src)[0] + ".o")
+        cmd = [nvcc(), *compile_flags, "-dc" if False else "-c", "-I", INCLUDE, "-I", CSRC,
+               "-o", obj, os.path.join(CSRC, src)]
+        res = subprocess.run(cmd, capture_output=True, text=True)
+        return src, obj, res
+
+    with ThreadPoolExecutor(max_workers=min(len(SOURCES), os.cpu_count() or 4)) as ex:
+        results = list(ex.map(compile_one, SOURCES))
+    log_txt = ""
+    for src, obj, res in results:
+        log_txt += f"==== {src}\n" + res.stderr
+        if res.returncode != 0:
+            sys.stderr.write(res.stdout + res.stderr)
+            raise RuntimeError(f"nvcc failed building {src}")
     tmp = LIB + f".tmp{os.getpid()}"
-    cmd = [nvcc(), *NVCC_FLAGS, "-I", INCLUDE, "-I", CSRC, "-o", tmp,
-           *[os.path.join(CSRC, s) for s in SOURCES]]
-    res = subprocess.run(cmd, capture_output=True, text=True)
+    link = [nvcc(), "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-Xcompiler", "-fPIC",
+            "-o", tmp, *[obj for _, obj, _ in results]]
+    res = subprocess.run(link, capture_output=True, text=True)
     if res.returncode != 0:
         sys.stderr.write(res.stdout + res.stderr)
-        raise RuntimeError("nvcc failed building libtridiag.so")
-    log = os.path.join(PKG, "csrc", "ptxas_last_build.txt")
-    with open(log, "w") as f:
-        f.write(res.stderr)
+        raise RuntimeError("nvcc link of libtridiag.so failed")
+    with open(os.path.join(PKG, "csrc", "ptxas_last_build.txt"), "w") as f:
+        f.write(log_txt)
     if verbose:
-        sys.stderr.write(res.stderr)
+        sys.stderr.write(log_txt)
     os.replace(tmp, LIB)
     return LIB
 

@@ -1,0 +1,66 @@
+// host_common.h -- host-side declarations shared by the translation units of
+// libtridiag.so (tridiag_api.cu and the per-(dtype, inner) kernel
+// instantiation units inst_*.cu, compiled in parallel).
+#pragma once
+
+#include <cuda.h>
+#include <cuda_runtime.h>
+#include <cudaTypedefs.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <map>
+#include <mutex>
+#include <tuple>
+
+#include "tridiag.h"
+
+namespace tdg_host {
+
+extern thread_local int g_last_launches;  // launches of the last call on this thread
+
+struct Layout {
+  int64_t es, ss;  // element stride, system stride (elements)
+};
+
+// Launch plan: kernel family and per-lane equation count R per (dtype, n, S).
+struct Plan {
+  bool cta;  // CTA kernels (W warps / system) or warp kernels
+  int R;
+  int W;     // cta only
+};
+Plan plan_for(int dtype, int64_t n, int64_t S = -1);
+
+int device_sms(int dev);
+int prefetch_mode();
+int tma_mode();
+int blocked_minb();
+PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
+
+std::mutex& occ_mutex();
+std::map<std::tuple<int, const void*, int, size_t>, int>& occ_cache();
+
+// Resident CTAs per SM of `kernel` (cached per device / kernel / size).
+template <typename K>
+int occupancy(int dev, K kernel, int threads, size_t smem) {
+  const void* key = reinterpret_cast<const void*>(kernel);
+  std::lock_guard<std::mutex> lk(occ_mutex());
+  auto& cache = occ_cache();
+  auto it = cache.find({dev, key, threads, smem});
+  if (it != cache.end()) return it->second;
+  if (smem > 48 * 1024) cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, kernel, threads, smem) != cudaSuccess) nb = 0;
+  cache[{dev, key, threads, smem}] = nb;
+  return nb;
+}
+
+// Enqueue one solve of S systems (n = padded size, nr = real size, k CR
+// levels) with the kernels of element type T and inner solver INNER.
+// Explicitly instantiated in inst_<f32|f64>_<pcr|rd>.cu.
+template <typename T, int INNER>
+cudaError_t dispatch_t(const void* a, const void* b, const void* c, const void* d, void* x,
+                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr,
+                       Layout L);
+
+}  // namespace tdg_host

@@ -1,0 +1,9 @@
+// Kernel instantiations of libtridiag.so for T = float, inner = RD
+// (one translation unit per combination so nvcc builds them in parallel).
+#include "launch.cuh"
+
+namespace tdg_host {
+template cudaError_t dispatch_t<float, tdg::kRD>(const void*, const void*, const void*, const void*,
+                                            void*, int64_t, int64_t, int, cudaStream_t, int,
+                                            int64_t, Layout);
+}  // namespace tdg_host

@@ -1,0 +1,203 @@
+// launch.cuh -- kernel launchers and dispatch of libtridiag.so (included by
+// the instantiation units inst_*.cu; see host_common.h).
+#pragma once
+
+#include "host_common.h"
+#include "tridiag_ileave.cuh"
+#include "tridiag_tma.cuh"
+
+namespace tdg_host {
+
+using tdg::ilog2c;
+
+template <typename T, int R, int INNER, int KB>
+cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                            int64_t S, int k, cudaStream_t st, int64_t n_real, Layout L) {
+  const int P = (int)(n / R);
+  const int G = std::max(8, 32 / P);
+  const int threads = G * P;
+  // 16-byte vector row segments when every row segment is 16-byte aligned
+  auto a16 = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) & 15) == 0; };
+  const int vec16 = a16(a) && a16(b) && a16(c) && a16(d) && a16(x) &&
+                    ((uint64_t)L.es * sizeof(T)) % 16 == 0 ? 1 : 0;
+  const size_t smem = (size_t)4 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
+  if (smem > 227 * 1024) return cudaErrorInvalidValue;
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = tdg::tdg_ileave_kernel<T, R, INNER, KB>;
+  const int occ = occupancy(dev, kern, threads, smem);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t tiles = (S + G - 1) / G;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)device_sms(dev) * occ));
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, ilog2c(P),
+                                              ilog2c(G), (int)n_real, c_pad, (long long)L.es, vec16);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
+template <typename T, int R, int INNER, int KB>
+cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                          int64_t S, int k, bool vec, cudaStream_t st, int64_t n_real, Layout L) {
+  if (L.ss == 1 && L.es != 1) return launch_ileave_k<T, R, INNER, KB>(a, b, c, d, x, n, S, k, st, n_real, L);
+  const int P = (int)(n / R);
+  const int log2P = ilog2c(P);
+  const int G = 32 / P;
+  const int wpb = 8;
+  const int threads = wpb * 32;
+  int dev = 0;
+  cudaGetDevice(&dev);
+  // vec: the contiguous power-of-two vector path; otherwise the general
+  // (scalar / strided / padded) instantiation
+  // The tuned register path (KB < 0, vector) lets ptxas choose (~127
+  // registers); every other instantiation asks for two CTAs per SM
+  // (TRIDIAG_BLOCKED_MINB=1 at run time selects the unconstrained build for
+  // the blocked inner instead, for A/B measurements).
+  auto kern = (KB < 0 && vec) ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
+            : (KB < 0)        ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>
+            : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
+                                         : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
+                  : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
+  const int occ = occupancy(dev, kern, threads, 0);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
+  const int pm = prefetch_mode();
+  const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
+                                           vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
+                                           (long long)L.ss);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
+// k >= log2 R: one register-path kernel for every such k; k < log2 R: the
+// blocked-inner kernel compiled for that k.
+template <typename T, int R, int INNER>
+cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
+  constexpr int LR = ilog2c(R);
+  if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+  switch (k) {
+    case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+    case 1: if constexpr (LR > 1) return launch_warp_k<T, R, INNER, 1>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
+    case 2: if constexpr (LR > 2) return launch_warp_k<T, R, INNER, 2>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
+    case 3: if constexpr (LR > 3) return launch_warp_k<T, R, INNER, 3>(a, b, c, d, x, n, S, k, vec, st, nr, L); break;
+  }
+  return cudaErrorInvalidValue;
+}
+
+// View one input array as [S*n/R rows][R columns] (64-byte rows), boxes of
+// min(P, 256) rows, 64-byte swizzle.
+template <typename T>
+bool make_row_map(CUtensorMap* m, const void* base, int64_t rows, int R, int box_rows) {
+  auto fn = encode_fn();
+  if (!fn) return false;
+  const cuuint64_t dims[2] = {(cuuint64_t)R, (cuuint64_t)rows};
+  const cuuint64_t strides[1] = {(cuuint64_t)R * sizeof(T)};
+  const cuuint32_t box[2] = {(cuuint32_t)R, (cuuint32_t)box_rows};
+  const cuuint32_t estr[2] = {1, 1};
+  const CUresult r = fn(m, sizeof(T) == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64,
+                        2, const_cast<void*>(base), dims, strides, box, estr,
+                        CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_64B,
+                        CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS;
+}
+
+template <typename T, int R, int W, int INNER>
+cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                           int64_t S, int k, cudaStream_t st, bool* used) {
+  *used = false;
+  const int P = 32 * W;
+  const int64_t rows = S * P;
+  if (rows >= (int64_t(1) << 31)) return cudaSuccess;
+  CUtensorMap mA, mB, mC, mD;
+  const int box = P > 256 ? 256 : P;
+  if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
+      !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box))
+    return cudaSuccess;
+  const size_t smem = tdg::cta_tma_smem_bytes<T>(R, W, INNER, k);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER>;
+  const int occ = occupancy(dev, kern, W * 32, smem);
+  if (occ <= 0) return cudaSuccess;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(mA, mB, mC, mD, x, (int)n, (long long)S, k);
+  g_last_launches = 1;
+  *used = true;
+  return cudaGetLastError();
+}
+
+template <typename T, int R, int W, int INNER>
+cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
+                       int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
+  if (vec && nr == n && L.es == 1 && L.ss == n && k >= ilog2c(R) && tma_mode()) {
+    bool used = false;
+    const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
+    if (used || e != cudaSuccess) return e;
+  }
+  const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  auto kern = k < ilog2c(R) ? tdg::tdg_cta_kernel<T, R, W, INNER, true>
+                             : tdg::tdg_cta_kernel<T, R, W, INNER, false>;
+  const int occ = occupancy(dev, kern, W * 32, smem);
+  if (occ <= 0) return cudaErrorInvalidConfiguration;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
+  const int pm = prefetch_mode();
+  const int pf = vec && (pm == 1 || pm == 2) ? 1 : 0;
+  const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  kern<<<(unsigned)grid, W * 32, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf,
+                                             (int)nr, c_pad, (long long)L.es, (long long)L.ss);
+  g_last_launches = 1;
+  return cudaGetLastError();
+}
+
+template <typename T, int INNER>
+cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const void* d_, void* x_,
+                       int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr,
+                       Layout L) {
+  const T* a = static_cast<const T*>(a_);
+  const T* b = static_cast<const T*>(b_);
+  const T* c = static_cast<const T*>(c_);
+  const T* d = static_cast<const T*>(d_);
+  T* x = static_cast<T*>(x_);
+  const Plan p = plan_for(dtype, n, S);
+  const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
+  auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
+  const bool vec = nr == n && L.es == 1 && ((uint64_t)L.ss * sizeof(T)) % tile == 0 && al(a) &&
+                   al(b) && al(c) && al(d) && al(x);
+  if (!p.cta) {
+    switch (p.R) {
+      case 1: return launch_warp<T, 1, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 2: return launch_warp<T, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_warp<T, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_warp<T, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 16:
+        if constexpr (sizeof(T) == 4) return launch_warp<T, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+        break;
+    }
+    return cudaErrorInvalidValue;
+  }
+  if constexpr (sizeof(T) == 4) {
+    switch (p.W) {
+      case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_cta<T, 16, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 16: return launch_cta<T, 16, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+    }
+  } else {
+    switch (p.W) {
+      case 2: return launch_cta<T, 8, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 4: return launch_cta<T, 8, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 8: return launch_cta<T, 8, 8, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+      case 16: return launch_cta<T, 8, 16, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
+    }
+  }
+  return cudaErrorInvalidValue;
+}
+
+
+}  // namespace tdg_host

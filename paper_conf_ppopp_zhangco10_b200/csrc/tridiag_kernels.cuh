@@ -19,6 +19,10 @@
 
 #include "tridiag_device.cuh"
 
+#ifndef TDG_BLOCKED_MINB
+#define TDG_BLOCKED_MINB 2
+#endif
+
 namespace tdg {
 
 // ============================================================================
@@ -48,11 +52,15 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
   inlane_backward<T, R>(a, b, c, d, kin, xprev);
 }
 
-template <typename T, int R, int INNER, int KB>
-__global__ void __launch_bounds__(256)
-tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
-                int n_real, T c_pad, long long es, long long ss) {
+// GEN = false: contiguous power-of-two systems with aligned pointers (vector
+// loads only).  GEN = true: the general path -- scalar loads, element / system
+// strides, padded (ragged) n -- compiled separately so the fast path carries
+// none of its registers.
+template <typename T, int R, int INNER, int KB, bool GEN>
+__device__ __forceinline__ void warp_kernel_body(
+    const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c, const T* d, T* x,
+    int n, long long S, int k, int log2P, int vec, int pf, int n_real, T c_pad, long long es,
+    long long ss) {
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -71,8 +79,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
     }
     const long long sys = s0 + sub;
     const bool valid = sys < S;
-    // general (scalar, strided and/or padded) path unless contiguous power of two
-    const bool ragged = n_real != n || es != 1;  // uniform
+    constexpr bool ragged = GEN;
     const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
@@ -99,6 +106,30 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
       else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
     }
   }
+}
+
+// KB < 0 (the register path of the tuned hybrids and CR): ptxas picks ~127
+// registers for 256 threads, two CTAs (16 warps) per SM.
+template <typename T, int R, int INNER, int KB, bool GEN>
+__global__ void __launch_bounds__(256)
+tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
+                const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
+                int n_real, T c_pad, long long es, long long ss) {
+  warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
+                                         es, ss);
+}
+
+// KB >= 0 (register-blocked inner: PCR, RD, large m) is latency bound with
+// one 8-warp CTA per SM at ~170 registers; asking for two CTAs (<= 128
+// registers; the few spills land in the otherwise unused L1) doubles the
+// warps that hide the shuffle / MUFU latency.
+template <typename T, int R, int INNER, int KB, bool GEN>
+__global__ void __launch_bounds__(256, R >= 8 ? TDG_BLOCKED_MINB : 1)
+tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
+                        const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
+                        int n_real, T c_pad, long long es, long long ss) {
+  warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
+                                         es, ss);
 }
 
 // ============================================================================
