@@ -1,0 +1,46 @@
+"""Small launches of every kernel family, for compute-sanitizer
+(racecheck / synccheck / memcheck / initcheck).  Checks results too."""
+import os
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import numpy as np  # noqa: E402
+import torch  # noqa: E402
+
+import oracle  # noqa: E402
+import paper_conf_ppopp_zhangco10_b200 as td  # noqa: E402
+from paper_conf_ppopp_zhangco10_b200 import inputs  # noqa: E402
+
+CASES = [
+    # (dtype, n, S, algo, m, layout)  -- one per kernel family
+    (torch.float32, 512, 40, "cr_pcr", 0, "contig"),     # warp kernel, register path
+    (torch.float32, 512, 40, "pcr", 0, "contig"),        # warp kernel, blocked inner
+    (torch.float32, 64, 40, "cr_rd", 16, "contig"),      # blocked RD
+    (torch.float32, 2048, 6, "cr_pcr", 0, "contig"),     # TMA CTA kernel
+    (torch.float32, 2048, 6, "cr_pcr", 1024, "contig"),  # CTA kernel, shared-memory inner
+    (torch.float64, 1024, 5, "cr_rd", 0, "contig"),      # TMA CTA kernel fp64
+    (torch.float32, 100, 33, "cr_pcr", 0, "contig"),     # ragged n (general path)
+    (torch.float32, 256, 30, "cr_pcr", 0, "column"),     # interleaved tile kernel
+    (torch.float32, 1024, 12, "cr", 0, "column"),        # CTA general strided path
+]
+
+only = sys.argv[1:] and int(sys.argv[1])
+bad = 0
+for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
+    if only not in ("", None) and idx != only:
+        continue
+    fam = "poi" if algo in ("rd", "cr_rd") else "dd"
+    a, b, c, d = inputs.generate(fam, S, n, dt, device="cuda")
+    if layout == "column":
+        views = [t.t().contiguous().t() for t in (a, b, c, d)]
+    else:
+        views = [a, b, c, d]
+    x = td.solve_batched(*views, algo=algo, switch_level=m)
+    torch.cuda.synchronize()
+    ref = oracle.thomas(*[t.cpu().numpy() for t in (a, b, c, d)])
+    e = float(np.max(oracle.normwise_error(x.contiguous().cpu().numpy(), ref)))
+    tol = 1e-4 if dt == torch.float32 else 1e-10
+    ok = e <= tol
+    bad += not ok
+    print(f"case {idx}: {dt} n={n} S={S} {algo} m={m} {layout}: err {e:.2e} {'ok' if ok else 'FAIL'}")
+sys.exit(1 if bad else 0)
