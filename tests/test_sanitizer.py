@@ -19,10 +19,8 @@ def test_compute_sanitizer(tool):
     torch = pytest.importorskip("torch")
     if not torch.cuda.is_available() or not os.path.exists(SAN):
         pytest.skip("needs a GPU and compute-sanitizer")
-    cmd = [SAN, "--tool", tool, "--error-exitcode", "3", sys.executable,
+    cmd = [SAN, "--tool", tool, "--target-processes", "all", "--error-exitcode", "3", sys.executable,
            os.path.join(ROOT, "tools", "sanitize_target.py")]
-    if tool == "initcheck":
-        cmd[1:1] = ["--track-unused-memory", "no"]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=1200, cwd=ROOT)
     out = r.stdout + r.stderr
     assert r.returncode == 0, out[-4000:]

@@ -24,10 +24,10 @@ CASES = [
     (torch.float32, 1024, 12, "cr", 0, "column"),        # CTA general strided path
 ]
 
-only = sys.argv[1:] and int(sys.argv[1])
+only = int(sys.argv[1]) if len(sys.argv) > 1 else None
 bad = 0
 for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
-    if only not in ("", None) and idx != only:
+    if only is not None and idx != only:
         continue
     fam = "poi" if algo in ("rd", "cr_rd") else "dd"
     a, b, c, d = inputs.generate(fam, S, n, dt, device="cuda")
