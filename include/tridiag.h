@@ -167,6 +167,20 @@ int tridiag_abi_version(void);
  * made on this thread (0 when S == 0).  For the bench's launch count. */
 int tridiag_last_launch_count(void);
 
+/*
+ * tridiag_phase_stamps -- diagnostic (the analogue of
+ * the paper's per-phase timing, Figs 8/11/13/15/16).  Only active
+ * when the process runs with TRIDIAG_PHASE_STAMPS=1: the warp kernels then
+ * record clock64() on lane 0 of warp 0 of every CTA at the phase boundaries
+ * of its first 4 system groups, as rows of 8 int64:
+ *   [0] start  [1] loads + in-lane CR forward  [2] tail chain
+ *   [3] lane-level CR + inner PCR/RD (or blocked inner)
+ *   [4] in-lane back-substitution  [5] store issued  [6..7] unused (0)
+ * Copies up to `cap` values of the last launch into host `out` (synchronous)
+ * and returns how many; 0 when inactive.
+ */
+int64_t tridiag_phase_stamps(int64_t* out, int64_t cap);
+
 #ifdef __cplusplus
 }
 #endif

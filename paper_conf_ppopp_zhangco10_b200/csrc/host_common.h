@@ -35,6 +35,9 @@ int device_sms(int dev);
 int prefetch_mode();
 int tma_mode();
 int blocked_minb();
+// Phase-stamp buffer for the next launch (nullptr unless TRIDIAG_PHASE_STAMPS=1;
+// diagnostic only: the one device allocation the library ever makes).
+long long* stamp_buffer(int64_t elems);
 PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 
 std::mutex& occ_mutex();

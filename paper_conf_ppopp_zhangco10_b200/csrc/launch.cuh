@@ -65,9 +65,10 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int pm = prefetch_mode();
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
+  long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
   kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
                                            vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
-                                           (long long)L.ss);
+                                           (long long)L.ss, stamps);
   g_last_launches = 1;
   return cudaGetLastError();
 }

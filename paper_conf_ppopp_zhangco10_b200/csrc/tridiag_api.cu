@@ -90,6 +90,29 @@ int blocked_minb() {
   return v;
 }
 
+// Phase stamps (diagnostic, NEXT f4): one device buffer per process, grown on
+// demand; tridiag_phase_stamps() copies the last launch's stamps back.
+namespace {
+std::mutex g_stamp_mu;
+long long* g_stamp_dev = nullptr;
+int64_t g_stamp_cap = 0, g_stamp_len = 0;
+}  // namespace
+long long* stamp_buffer(int64_t elems) {
+  static const int on = env_int("TRIDIAG_PHASE_STAMPS", 0);
+  if (!on) return nullptr;
+  std::lock_guard<std::mutex> lk(g_stamp_mu);
+  if (elems > g_stamp_cap) {
+    if (g_stamp_dev) cudaFree(g_stamp_dev);
+    g_stamp_dev = nullptr;
+    g_stamp_cap = 0;
+    if (cudaMalloc(&g_stamp_dev, elems * sizeof(long long)) != cudaSuccess) return nullptr;
+    g_stamp_cap = elems;
+  }
+  cudaMemset(g_stamp_dev, 0, elems * sizeof(long long));
+  g_stamp_len = elems;
+  return g_stamp_dev;
+}
+
 // R per lane from the plan sweep (profiles/r01_tune_plan.md): on HBM-scale
 // batches the widest register block that fits (16 fp32 / 8 fp64 equations per
 // lane) is fastest at every n, and systems with n <= 32 use 4 lanes.  Small
@@ -230,6 +253,14 @@ extern "C" {
 int tridiag_abi_version(void) { return TRIDIAG_ABI_VERSION; }
 
 int tridiag_last_launch_count(void) { return g_last_launches; }
+
+int64_t tridiag_phase_stamps(int64_t* out, int64_t cap) {
+  std::lock_guard<std::mutex> lk(g_stamp_mu);
+  if (!g_stamp_dev || !out || cap <= 0) return 0;
+  const int64_t len = std::min<int64_t>(cap, g_stamp_len);
+  if (cudaMemcpy(out, g_stamp_dev, len * sizeof(long long), cudaMemcpyDeviceToHost) != cudaSuccess) return 0;
+  return len;
+}
 
 const char* tridiag_status_string(int status) {
   switch (status) {

@@ -28,17 +28,32 @@ namespace tdg {
 // ============================================================================
 // Warp kernel.
 // ============================================================================
+// Phase stamps: the paper times its solvers phase
+// by phase (Figs 8, 11, 13, 15, 16).  When the launch passes a
+// stamp buffer, lane 0 of warp 0 of every CTA records clock64() at the phase
+// boundaries of its first kStampSystems system groups (no effect otherwise).
+constexpr int kStampSystems = 4;
+constexpr int kStampSlots = 8;
+struct Stamp {
+  long long* p = nullptr;
+  __device__ __forceinline__ void mark(int slot) const {
+    if (p != nullptr && (threadIdx.x & 31) == 0) p[slot] = clock64();
+  }
+};
+
 // KB < 0: k >= LR (all in-lane levels; m <= P, lane-level inner solve).
 // KB >= 0: k == KB < LR (m = P * (R >> KB) > P, register-blocked inner solve).
 template <typename T, int R, int INNER, int KB>
 __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&d)[R], int k,
-                                           int ls, int P) {
+                                           int ls, int P, Stamp st = Stamp()) {
   constexpr int LR = ilog2c(R);
   constexpr int kin = KB < 0 ? LR : KB;
   inlane_forward_interior<T, R>(a, b, c, d, kin);
+  st.mark(1);
   Heads<T, R> H;
   heads_from_next_lane<T, R>(a, b, c, d, kin, P, ls == P - 1, H);
   inlane_tail_chain<T, R>(a, b, c, d, kin, H);
+  st.mark(2);
   if constexpr (KB < 0) {
     d[R - 1] = lane_level_solve<T, INNER>(a[R - 1], b[R - 1], c[R - 1], d[R - 1], k - LR, ls, P);
   } else {
@@ -47,9 +62,11 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
     if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
     else blocked_rd<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
   }
+  st.mark(3);
   T xprev = __shfl_up_sync(kFull, d[R - 1], 1, P);
   if (ls == 0) xprev = T(0);
   inlane_backward<T, R>(a, b, c, d, kin, xprev);
+  st.mark(4);
 }
 
 // GEN = false: contiguous power-of-two systems with aligned pointers (vector
@@ -60,7 +77,7 @@ template <typename T, int R, int INNER, int KB, bool GEN>
 __device__ __forceinline__ void warp_kernel_body(
     const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c, const T* d, T* x,
     int n, long long S, int k, int log2P, int vec, int pf, int n_real, T c_pad, long long es,
-    long long ss) {
+    long long ss, long long* stamps) {
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -69,7 +86,12 @@ __device__ __forceinline__ void warp_kernel_body(
   const int sub = lane >> log2P;
   const int ls = lane & (P - 1);
   const long long step = (long long)gridDim.x * wpb * G;
-  for (long long s0 = ((long long)blockIdx.x * wpb + warp) * G; s0 < S; s0 += step) {
+  int iter = 0;
+  for (long long s0 = ((long long)blockIdx.x * wpb + warp) * G; s0 < S; s0 += step, ++iter) {
+    Stamp stp;
+    if (stamps != nullptr && warp == 0 && iter < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + iter) * kStampSlots;
+    stp.mark(0);
     if (pf && lane < 4 && s0 + step < S) {
       // lanes 0..3 prefetch array a, b, c, d of this warp's next group
       const long long nx = s0 + step;
@@ -100,11 +122,12 @@ __device__ __forceinline__ void warp_kernel_body(
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
-    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
+    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp);
     if (valid) {
       if (!ragged) store_block<T, R>(x + off, rd, vec);
       else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
     }
+    stp.mark(5);
   }
 }
 
@@ -114,9 +137,9 @@ template <typename T, int R, int INNER, int KB, bool GEN>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
-                int n_real, T c_pad, long long es, long long ss) {
+                int n_real, T c_pad, long long es, long long ss, long long* stamps) {
   warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
-                                         es, ss);
+                                         es, ss, stamps);
 }
 
 // KB >= 0 (register-blocked inner: PCR, RD, large m) is latency bound with
@@ -127,9 +150,9 @@ template <typename T, int R, int INNER, int KB, bool GEN>
 __global__ void __launch_bounds__(256, R >= 8 ? TDG_BLOCKED_MINB : 1)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
-                        int n_real, T c_pad, long long es, long long ss) {
+                        int n_real, T c_pad, long long es, long long ss, long long* stamps) {
   warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
-                                         es, ss);
+                                         es, ss, stamps);
 }
 
 // ============================================================================

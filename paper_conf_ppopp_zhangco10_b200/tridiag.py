@@ -68,6 +68,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_abi_version.restype = I
         L.tridiag_last_launch_count.argtypes = []
         L.tridiag_last_launch_count.restype = I
+        L.tridiag_phase_stamps.argtypes = [P, I64]
+        L.tridiag_phase_stamps.restype = I64
         _lib = L
         return L
 
@@ -114,6 +116,14 @@ def abi_version() -> int:
 
 def last_launch_count() -> int:
     return int(load().tridiag_last_launch_count())
+
+
+def phase_stamps(cap: int = 1 << 20):
+    """Per-phase clock64() stamps of the last launch (TRIDIAG_PHASE_STAMPS=1
+    only), as an (rows, 8) int64 tensor; empty when inactive."""
+    buf = torch.zeros(cap, dtype=torch.int64)
+    n = int(load().tridiag_phase_stamps(buf.data_ptr(), cap))
+    return buf[: n - n % 8].view(-1, 8)
 
 
 def solve_batched_raw(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, n, num_systems, dtype, algo,
