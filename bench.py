@@ -52,6 +52,9 @@ def parse():
     p.add_argument("--family", default="dd")
     p.add_argument("--no-extras", action="store_true", help="skip per-algorithm table, e2e and cpu baseline")
     p.add_argument("--cpu-seconds", type=float, default=8.0, help="wall budget of the cpu_baseline leg")
+    p.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
+                   help="process group for the post-timing reductions (gloo: harness tests with "
+                        "several ranks on one GPU)")
     return p.parse_args()
 
 
@@ -278,9 +281,14 @@ def main():
 
     rank, local, world = dist_env()
     args.gpus = world
-    torch.cuda.set_device(local)
+    ndev = torch.cuda.device_count()
+    dev = local if local < ndev else local % ndev  # (>1 rank per GPU only for harness tests)
+    torch.cuda.set_device(dev)
     if world > 1:
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if args.dist_backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", dev))
+        else:
+            dist.init_process_group(args.dist_backend)
     td.load(build_if_missing=False)
     dt = torch.float32 if args.dtype == "f32" else torch.float64
     T = 4 if args.dtype == "f32" else 8
@@ -293,7 +301,7 @@ def main():
     a, b, c, d = inputs.generate(args.family, S, n, dt, s0=s0, device="cuda")
     x = torch.empty_like(d)
     stream = torch.cuda.Stream()
-    sampler = ClockSampler(local)
+    sampler = ClockSampler(dev)
 
     # warm-up, then the timed region: barrier + sync on both sides, max over ranks
     with torch.cuda.stream(stream):
