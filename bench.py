@@ -42,7 +42,8 @@ def parse():
     p.add_argument("--steps", type=int, default=200)
     p.add_argument("--warmup", type=int, default=20)
     p.add_argument("--impl", default="b200", choices=["b200", "reference"])
-    p.add_argument("--n", type=int, default=512)
+    p.add_argument("--system-size", dest="n", type=int, default=512,
+                   help="equations per system (named so torchrun does not claim it)")
     p.add_argument("--systems", type=int, default=131072, help="systems per GPU (weak scaling)")
     p.add_argument("--total-systems", type=int, default=0,
                    help="strong scaling: split this many systems over the ranks (C4: 1048576 x n=256)")
