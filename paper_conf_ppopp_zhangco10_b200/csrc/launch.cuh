@@ -58,7 +58,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
             : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
                                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
                   : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
-  const int occ = occupancy(dev, kern, threads, 0);
+  const int occ = occupancy(dev, kern, threads,
+                            vec ? 0 : (size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T));
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
@@ -66,7 +67,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
-  kern<<<(unsigned)grid, threads, 0, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
+  const size_t smem = vec ? 0 : (size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T);
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
                                            vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
                                            (long long)L.ss, stamps);
   g_last_launches = 1;
@@ -139,7 +141,8 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
     const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
     if (used || e != cudaSuccess) return e;
   }
-  const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k);
+  const bool staged = (nr != n || !vec) && L.es == 1;
+  const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k, staged);
   int dev = 0;
   cudaGetDevice(&dev);
   auto kern = k < ilog2c(R) ? tdg::tdg_cta_kernel<T, R, W, INNER, true>

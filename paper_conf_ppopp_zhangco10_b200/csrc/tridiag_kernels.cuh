@@ -69,6 +69,69 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
   st.mark(4);
 }
 
+// ---- warp-staged general path (contiguous rows of any length / alignment) ----
+// Per-warp shared tile of 32R elements per array (the warp's G systems of
+// n_pad = P R equations, back to back), element q at q + (q >> 5).
+template <typename T, int R>
+__host__ __device__ constexpr int warp_tile_elems() { return 32 * R + R + 1; }
+template <typename T, int R>
+__device__ __forceinline__ T* warp_tile(int warp) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  return reinterpret_cast<T*>(smem_raw) + (size_t)warp * 4 * warp_tile_elems<T, R>();
+}
+__device__ __forceinline__ int wt_off(int q) { return q + (q >> 5); }
+
+template <typename T, int R>
+__device__ __forceinline__ void staged_load(const T* a, const T* b, const T* c, const T* d,
+                                            long long s0, long long S, long long ss, int n_pad,
+                                            int n_real, T c_pad, int G, int lane, int sub,
+                                            T (&ra)[R], T (&rb)[R], T (&rc)[R], T (&rd)[R],
+                                            T* tile) {
+  constexpr int TE = warp_tile_elems<T, R>();
+  T* tA = tile;
+  T* tB = tile + TE;
+  T* tC = tile + 2 * TE;
+  T* tD = tile + 3 * TE;
+  for (int g = 0; g < G; ++g) {
+    const long long sys = s0 + g;
+    const bool ok = sys < S;
+    const size_t base = (size_t)sys * (size_t)ss;
+    for (int i = lane; i < n_pad; i += 32) {
+      const int o = wt_off(g * n_pad + i);
+      const bool v = ok && i < n_real;
+      tA[o] = v ? a[base + i] : T(0);
+      tB[o] = v ? b[base + i] : T(1);
+      tC[o] = v ? (i == n_real - 1 ? c_pad : c[base + i]) : c_pad;
+      tD[o] = v ? d[base + i] : T(0);
+    }
+  }
+  __syncwarp();
+#pragma unroll
+  for (int t = 0; t < R; ++t) {
+    const int o = wt_off(lane * R + t);
+    ra[t] = tA[o]; rb[t] = tB[o]; rc[t] = tC[o]; rd[t] = tD[o];
+  }
+  (void)sub;
+  __syncwarp();
+}
+
+template <typename T, int R>
+__device__ __forceinline__ void staged_store(T* x, long long s0, long long S, long long ss,
+                                             int n_pad, int n_real, int G, int lane,
+                                             const T (&rd)[R], T* tile) {
+  T* tD = tile + 3 * warp_tile_elems<T, R>();
+#pragma unroll
+  for (int t = 0; t < R; ++t) tD[wt_off(lane * R + t)] = rd[t];
+  __syncwarp();
+  for (int g = 0; g < G; ++g) {
+    const long long sys = s0 + g;
+    if (sys >= S) break;
+    const size_t base = (size_t)sys * (size_t)ss;
+    for (int i = lane; i < n_real; i += 32) x[base + i] = tD[wt_off(g * n_pad + i)];
+  }
+  __syncwarp();
+}
+
 // GEN = false: contiguous power-of-two systems with aligned pointers (vector
 // loads only).  GEN = true: the general path -- scalar loads, element / system
 // strides, padded (ragged) n -- compiled separately so the fast path carries
@@ -101,31 +164,35 @@ __device__ __forceinline__ void warp_kernel_body(
     }
     const long long sys = s0 + sub;
     const bool valid = sys < S;
-    constexpr bool ragged = GEN;
     const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
-    if (valid && !ragged) {
-      load_block<T, R, true>(a + off, ra, vec);
-      load_block<T, R, true>(b + off, rb, vec);
-      load_block<T, R, true>(c + off, rc, vec);
-      load_block<T, R, false>(d + off, rd, vec);
-    } else if (valid) {
-      load_ragged<T, R>(a + sbase, es, ls * R, n_real, ra, T(0), T(0), false);
-      load_ragged<T, R>(b + sbase, es, ls * R, n_real, rb, T(1), T(0), false);
-      load_ragged<T, R>(c + sbase, es, ls * R, n_real, rc, c_pad, c_pad, true);
-      load_ragged<T, R>(d + sbase, es, ls * R, n_real, rd, T(0), T(0), false);
-    } else {
+    if constexpr (!GEN) {
+      if (valid) {
+        load_block<T, R, true>(a + off, ra, vec);
+        load_block<T, R, true>(b + off, rb, vec);
+        load_block<T, R, true>(c + off, rc, vec);
+        load_block<T, R, false>(d + off, rd, vec);
+      } else {
 #pragma unroll
-      for (int i = 0; i < R; ++i) { ra[i] = T(0); rb[i] = T(1); rc[i] = T(0); rd[i] = T(0); }
+        for (int i = 0; i < R; ++i) { ra[i] = T(0); rb[i] = T(1); rc[i] = T(0); rd[i] = T(0); }
+      }
+    } else {
+      // General contiguous rows (ragged n, misaligned or pitched): the warp
+      // reads its G systems with coalesced, lane-consecutive loads into a
+      // per-warp shared tile (padded one element per 32, so the lane-blocked
+      // reads below are bank-conflict free), padding included.
+      staged_load<T, R>(a, b, c, d, s0, S, ss, n, n_real, c_pad, G, lane, sub, ra, rb, rc, rd,
+                        warp_tile<T, R>(warp));
     }
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp);
-    if (valid) {
-      if (!ragged) store_block<T, R>(x + off, rd, vec);
-      else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
+    if constexpr (!GEN) {
+      if (valid) store_block<T, R>(x + off, rd, vec);
+    } else {
+      staged_store<T, R>(x, s0, S, ss, n, n_real, G, lane, rd, warp_tile<T, R>(warp));
     }
     stp.mark(5);
   }
@@ -342,7 +409,11 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       prefetch_l2(base + (size_t)(sys + gridDim.x) * n + (size_t)warp * 32 * R,
                   (uint32_t)(32 * R * sizeof(T)));
     }
-    const bool ragged = n_real != n || es != 1;
+    const bool ragged = n_real != n || es != 1 || !vec;
+    // contiguous rows (any length / alignment / pitch): CTA-cooperative
+    // coalesced loads through a padded shared tile; element-strided rows
+    // (interleaved layouts with n > 32R) fall back to scalar loads.
+    const bool staged = ragged && es == 1;
     const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
@@ -351,6 +422,27 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       load_block<T, R, true>(b + off, rb, vec);
       load_block<T, R, true>(c + off, rc, vec);
       load_block<T, R, false>(d + off, rd, vec);
+    } else if (staged) {
+      const int TE = n + (n >> 5) + 1;
+      T* tA = work;
+      T* tB = work + TE;
+      T* tC = work + 2 * TE;
+      T* tD = work + 3 * TE;
+      for (int i = ls; i < n; i += P) {
+        const int o = wt_off(i);
+        const bool v = i < n_real;
+        tA[o] = v ? a[sbase + i] : T(0);
+        tB[o] = v ? b[sbase + i] : T(1);
+        tC[o] = v ? (i == n_real - 1 ? c_pad : c[sbase + i]) : c_pad;
+        tD[o] = v ? d[sbase + i] : T(0);
+      }
+      __syncthreads();
+#pragma unroll
+      for (int t = 0; t < R; ++t) {
+        const int o = wt_off(ls * R + t);
+        ra[t] = tA[o]; rb[t] = tB[o]; rc[t] = tC[o]; rd[t] = tD[o];
+      }
+      __syncthreads();  // the tile is reused by the heads / survivor regions
     } else {
       load_ragged<T, R>(a + sbase, es, ls * R, n_real, ra, T(0), T(0), false);
       load_ragged<T, R>(b + sbase, es, ls * R, n_real, rb, T(1), T(0), false);
@@ -392,15 +484,24 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       xprev = ls > 0 ? X[ls * q - 1] : T(0);
     }
     inlane_backward<T, R>(ra, rb, rc, rd, kin, xprev);
-    if (!ragged) store_block<T, R>(x + off, rd, vec);
-    else store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
+    if (!ragged) {
+      store_block<T, R>(x + off, rd, vec);
+    } else if (staged) {
+      __syncthreads();  // every thread is done with the survivor regions
+      T* tD = work + 3 * (n + (n >> 5) + 1);
+#pragma unroll
+      for (int t = 0; t < R; ++t) tD[wt_off(ls * R + t)] = rd[t];
+      __syncthreads();
+      for (int i = ls; i < n_real; i += P) x[sbase + i] = tD[wt_off(i)];
+    } else {
+      store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
+    }
     __syncthreads();  // shared memory is reused by the next system
   }
 }
 
-// Shared-memory bytes of tdg_cta_kernel for a given k.
 template <typename T>
-inline size_t cta_smem_bytes(int R, int W, int inner, int k) {
+inline size_t cta_smem_bytes_core(int R, int W, int inner, int k) {
   const int P = 32 * W;
   const int LR = ilog2c(R);
   const int LRH = LR > 0 ? LR : 1;
@@ -416,6 +517,16 @@ inline size_t cta_smem_bytes(int R, int W, int inner, int k) {
     e += inner_region_elems(inner, m);
   }
   return (size_t)e * sizeof(T);
+}
+
+// Shared-memory bytes of tdg_cta_kernel for a given k (staged: room for the
+// coalesced staging tile of the general path, 4 (n + n/32 + 1) elements).
+template <typename T>
+inline size_t cta_smem_bytes(int R, int W, int inner, int k, bool staged = false) {
+  const size_t base = cta_smem_bytes_core<T>(R, W, inner, k);
+  const int64_t n = 32LL * W * R;
+  const size_t tile = (size_t)(W * (ilog2c(R) > 0 ? ilog2c(R) : 1) * 4 + 4 * (n + (n >> 5) + 1)) * sizeof(T);
+  return staged && tile > base ? tile : base;
 }
 
 }  // namespace tdg
