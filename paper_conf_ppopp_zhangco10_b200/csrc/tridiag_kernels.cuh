@@ -81,10 +81,13 @@ __device__ __forceinline__ T* warp_tile(int warp) {
 }
 __device__ __forceinline__ int wt_off(int q) { return q + (q >> 5); }
 
+// The warp's tile holds 32R elements per array, so every lane moves exactly R
+// of them: element q = lane + 32 j (j < R, unrolled so all 4R loads are in
+// flight together) is equation i = q mod n_pad of system s0 + q / n_pad.
 template <typename T, int R>
 __device__ __forceinline__ void staged_load(const T* a, const T* b, const T* c, const T* d,
                                             long long s0, long long S, long long ss, int n_pad,
-                                            int n_real, T c_pad, int G, int lane, int sub,
+                                            int n_real, T c_pad, int log2n, int lane,
                                             T (&ra)[R], T (&rb)[R], T (&rc)[R], T (&rd)[R],
                                             T* tile) {
   constexpr int TE = warp_tile_elems<T, R>();
@@ -92,18 +95,23 @@ __device__ __forceinline__ void staged_load(const T* a, const T* b, const T* c, 
   T* tB = tile + TE;
   T* tC = tile + 2 * TE;
   T* tD = tile + 3 * TE;
-  for (int g = 0; g < G; ++g) {
+  T va[R], vb[R], vc[R], vd[R];
+#pragma unroll
+  for (int j = 0; j < R; ++j) {
+    const int q = lane + 32 * j;
+    const int g = q >> log2n, i = q & (n_pad - 1);
     const long long sys = s0 + g;
-    const bool ok = sys < S;
-    const size_t base = (size_t)sys * (size_t)ss;
-    for (int i = lane; i < n_pad; i += 32) {
-      const int o = wt_off(g * n_pad + i);
-      const bool v = ok && i < n_real;
-      tA[o] = v ? a[base + i] : T(0);
-      tB[o] = v ? b[base + i] : T(1);
-      tC[o] = v ? (i == n_real - 1 ? c_pad : c[base + i]) : c_pad;
-      tD[o] = v ? d[base + i] : T(0);
-    }
+    const bool v = sys < S && i < n_real;
+    const size_t e = (size_t)sys * (size_t)ss + i;
+    va[j] = v ? a[e] : T(0);
+    vb[j] = v ? b[e] : T(1);
+    vc[j] = v ? (i == n_real - 1 ? c_pad : c[e]) : c_pad;
+    vd[j] = v ? d[e] : T(0);
+  }
+#pragma unroll
+  for (int j = 0; j < R; ++j) {
+    const int o = wt_off(lane + 32 * j);
+    tA[o] = va[j]; tB[o] = vb[j]; tC[o] = vc[j]; tD[o] = vd[j];
   }
   __syncwarp();
 #pragma unroll
@@ -111,23 +119,23 @@ __device__ __forceinline__ void staged_load(const T* a, const T* b, const T* c, 
     const int o = wt_off(lane * R + t);
     ra[t] = tA[o]; rb[t] = tB[o]; rc[t] = tC[o]; rd[t] = tD[o];
   }
-  (void)sub;
   __syncwarp();
 }
 
 template <typename T, int R>
 __device__ __forceinline__ void staged_store(T* x, long long s0, long long S, long long ss,
-                                             int n_pad, int n_real, int G, int lane,
+                                             int n_pad, int n_real, int log2n, int lane,
                                              const T (&rd)[R], T* tile) {
   T* tD = tile + 3 * warp_tile_elems<T, R>();
 #pragma unroll
   for (int t = 0; t < R; ++t) tD[wt_off(lane * R + t)] = rd[t];
   __syncwarp();
-  for (int g = 0; g < G; ++g) {
+#pragma unroll
+  for (int j = 0; j < R; ++j) {
+    const int q = lane + 32 * j;
+    const int g = q >> log2n, i = q & (n_pad - 1);
     const long long sys = s0 + g;
-    if (sys >= S) break;
-    const size_t base = (size_t)sys * (size_t)ss;
-    for (int i = lane; i < n_real; i += 32) x[base + i] = tD[wt_off(g * n_pad + i)];
+    if (sys < S && i < n_real) x[(size_t)sys * (size_t)ss + i] = tD[wt_off(q)];
   }
   __syncwarp();
 }
@@ -182,8 +190,8 @@ __device__ __forceinline__ void warp_kernel_body(
       // reads its G systems with coalesced, lane-consecutive loads into a
       // per-warp shared tile (padded one element per 32, so the lane-blocked
       // reads below are bank-conflict free), padding included.
-      staged_load<T, R>(a, b, c, d, s0, S, ss, n, n_real, c_pad, G, lane, sub, ra, rb, rc, rd,
-                        warp_tile<T, R>(warp));
+      staged_load<T, R>(a, b, c, d, s0, S, ss, n, n_real, c_pad, log2P + ilog2c(R), lane, ra, rb,
+                        rc, rd, warp_tile<T, R>(warp));
     }
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
@@ -192,7 +200,7 @@ __device__ __forceinline__ void warp_kernel_body(
     if constexpr (!GEN) {
       if (valid) store_block<T, R>(x + off, rd, vec);
     } else {
-      staged_store<T, R>(x, s0, S, ss, n, n_real, G, lane, rd, warp_tile<T, R>(warp));
+      staged_store<T, R>(x, s0, S, ss, n, n_real, log2P + ilog2c(R), lane, rd, warp_tile<T, R>(warp));
     }
     stp.mark(5);
   }
@@ -428,13 +436,20 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
       T* tB = work + TE;
       T* tC = work + 2 * TE;
       T* tD = work + 3 * TE;
-      for (int i = ls; i < n; i += P) {
-        const int o = wt_off(i);
+      T va[R], vb[R], vc[R], vd[R];
+#pragma unroll
+      for (int j = 0; j < R; ++j) {  // element ls + P j: all 4R loads in flight
+        const int i = ls + P * j;
         const bool v = i < n_real;
-        tA[o] = v ? a[sbase + i] : T(0);
-        tB[o] = v ? b[sbase + i] : T(1);
-        tC[o] = v ? (i == n_real - 1 ? c_pad : c[sbase + i]) : c_pad;
-        tD[o] = v ? d[sbase + i] : T(0);
+        va[j] = v ? a[sbase + i] : T(0);
+        vb[j] = v ? b[sbase + i] : T(1);
+        vc[j] = v ? (i == n_real - 1 ? c_pad : c[sbase + i]) : c_pad;
+        vd[j] = v ? d[sbase + i] : T(0);
+      }
+#pragma unroll
+      for (int j = 0; j < R; ++j) {
+        const int o = wt_off(ls + P * j);
+        tA[o] = va[j]; tB[o] = vb[j]; tC[o] = vc[j]; tD[o] = vd[j];
       }
       __syncthreads();
 #pragma unroll
@@ -492,7 +507,11 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
 #pragma unroll
       for (int t = 0; t < R; ++t) tD[wt_off(ls * R + t)] = rd[t];
       __syncthreads();
-      for (int i = ls; i < n_real; i += P) x[sbase + i] = tD[wt_off(i)];
+#pragma unroll
+      for (int j = 0; j < R; ++j) {
+        const int i = ls + P * j;
+        if (i < n_real) x[sbase + i] = tD[wt_off(i)];
+      }
     } else {
       store_ragged<T, R>(x + sbase, es, ls * R, n_real, rd);
     }
