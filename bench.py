@@ -394,6 +394,43 @@ def main():
                 per_algo[key] = {"systems_per_s": sps, "gbs_per_gpu": gbs, "frac_of_peak": gbs / peak,
                                  "family": fam}
         line["per_algo"] = per_algo
+        # the other BASELINE.json configs (CR+PCR at the tuned m, this rank's GPU):
+        # C3 ADI-style 4096 x 4096 (row sweep contiguous, column sweep interleaved),
+        # C4 2^20 x 256 on one GPU, C5's largest system n = 8192.
+        del a, b, c, d, x
+        torch.cuda.empty_cache()
+        other = {}
+        for name, dts, nn, SS, layout in (("c3_f32_4096x4096_rows", "f32", 4096, 4096, "rows"),
+                                          ("c3_f32_4096x4096_columns", "f32", 4096, 4096, "cols"),
+                                          ("c3_f64_4096x4096_rows", "f64", 4096, 4096, "rows"),
+                                          ("c4_f32_1048576x256", "f32", 256, 1 << 20, "rows"),
+                                          ("c5_f32_16384x8192", "f32", 8192, 16384, "rows")):
+            dtt = torch.float32 if dts == "f32" else torch.float64
+            TT = 4 if dts == "f32" else 8
+            sets = []
+            nsets = max(1, -(-4 * 126 * 2**20 // (5 * nn * SS * TT)))
+            for kk in range(nsets):
+                g = inputs.generate("dd", SS, nn, dtt, s0=kk * SS, device="cuda")
+                if layout == "cols":
+                    g = [t.t().contiguous().t() for t in g]
+                sets.append((*g, torch.empty_like(g[3])))
+            steps = max(5, args.steps // 10)
+            for i in range(3):
+                td.solve_batched(*sets[i % nsets], algo="cr_pcr", stream=stream)
+            torch.cuda.synchronize()
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record(stream)
+            for i in range(steps):
+                td.solve_batched(*sets[i % nsets], algo="cr_pcr", stream=stream)
+            e1.record(stream)
+            torch.cuda.synchronize()
+            tt = reduce_max(e0.elapsed_time(e1) / 1e3 / steps)
+            gbs = 5 * nn * TT * SS / tt / 1e9
+            other[name] = {"systems_per_s_per_gpu": SS / tt, "gbs_per_gpu": gbs,
+                           "frac_of_peak": gbs / peak, "layout": layout, "algo": "cr_pcr"}
+            del sets
+            torch.cuda.empty_cache()
+        line["other_configs"] = other
         if rank == 0:
             line["cpu_baseline"] = cpu_baseline(n, S, dt, args.family, args.cpu_seconds)
         line["paper_context"] = {"gtx280_cr_pcr_512x512_ms": 0.422,
