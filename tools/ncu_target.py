@@ -19,9 +19,12 @@ p.add_argument("--algo", default="cr_pcr")
 p.add_argument("--m", type=int, default=0)
 p.add_argument("--family", default="dd")
 p.add_argument("--reps", type=int, default=4)
+p.add_argument("--layout", default="rows", choices=["rows", "cols", "ragged"])
 a = p.parse_args()
 dt = torch.float32 if a.dtype == "f32" else torch.float64
 A, B, C, D = inputs.generate(a.family, a.systems, a.n, dt, device="cuda")
+if a.layout == "cols":
+    A, B, C, D = [t.t().contiguous().t() for t in (A, B, C, D)]
 X = torch.empty_like(D)
 torch.cuda.synchronize()
 for _ in range(a.reps):
