@@ -18,7 +18,8 @@ cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x
   const int threads = G * P;
   // 16-byte vector row segments when every row segment is 16-byte aligned
   auto a16 = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) & 15) == 0; };
-  const int vec16 = a16(a) && a16(b) && a16(c) && a16(d) && a16(x) &&
+  // (each thread moves R / V row segments: needs R >= V = 16 / sizeof(T))
+  const int vec16 = R * sizeof(T) >= 16 && a16(a) && a16(b) && a16(c) && a16(d) && a16(x) &&
                     ((uint64_t)L.es * sizeof(T)) % 16 == 0 ? 1 : 0;
   const size_t smem = (size_t)4 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
   if (smem > 227 * 1024) return cudaErrorInvalidValue;
