@@ -36,7 +36,14 @@ typedef enum {
     TRIDIAG_PCR = 1,    /* P:L313-386, Fig 2                                    */
     TRIDIAG_RD = 2,     /* P:L387-421, Fig 3 (Egecioglu scan form of Stone's RD) */
     TRIDIAG_CR_PCR = 3, /* P:L572-581, Fig 4: CR to m equations, PCR, CR back   */
-    TRIDIAG_CR_RD = 4   /* P:L572-581, Fig 4: CR to m equations, RD, CR back    */
+    TRIDIAG_CR_RD = 4,  /* P:L572-581, Fig 4: CR to m equations, RD, CR back    */
+    /* Not one of the paper's five: overflow-free recursive doubling in LU
+     * form (the paper's RD overflows on dominant rows,
+     * P:L1219-1236, and it cites Stone [27]): three Hillis-Steele scans --
+     * power-of-two-rescaled 2x2 continuant products for the LU pivots, then
+     * the forward and backward affine recurrences, which contract on
+     * diagonally dominant rows.  n <= 512 (fp32) / 256 (fp64). */
+    TRIDIAG_RD_STONE = 5
 } tridiag_algo;
 
 /* Status codes.  0 = enqueued.  Negative = argument error, nothing enqueued.

@@ -28,6 +28,10 @@ Functions (all take (S, n) C-contiguous arrays; fp64 unless noted):
                      Fig 4).  Pinned by: Fig 4 dataflow, endpoint identities
                      (m=2 == CR, m=n == PCR/RD bitwise, Fig 17),
                      step counts (reading R13), dgtsv.
+* ``rd_stone``    -- overflow-free RD in LU form (NEXT f3): rescaled 2x2
+                     continuant scan + two affine scans.  Pinned by: dgtsv on
+                     DD / KM (where the paper's RD overflows), dense gesv,
+                     3 log2 n + 4 steps, no overflow at n = 8192.
 * ``thomas_mt``   -- the paper's MT CPU solver: threads solving
                      whole systems; the timed cpu_baseline.
 
@@ -84,7 +88,7 @@ def _load():
             f = getattr(lib, f"oracle_thomas_mt_{sfx}")
             f.argtypes = [P, P, P, P, P, I64, I64, ctypes.c_int]
             f.restype = ctypes.c_int
-            for name in ("cr", "pcr", "rd"):
+            for name in ("cr", "pcr", "rd", "rd_stone"):
                 f = getattr(lib, f"oracle_{name}_{sfx}")
                 f.argtypes = [P, P, P, P, P, I64, I64, I64P, I64P, I64, I64P]
                 f.restype = ctypes.c_int
@@ -191,6 +195,14 @@ def rd(a, b, c, d, dtype=np.float64, log_events=False, log_cap=1 << 18):
     return _run_stepped("rd", a, b, c, d, dtype, (), log_events, log_cap)
 
 
+def rd_stone(a, b, c, d, dtype=np.float64):
+    """Overflow-free RD in LU form (NEXT f3; Stone [27] as cited at P:L387-389):
+    three Hillis-Steele scans -- rescaled 2x2 continuant products for the
+    pivots, forward and backward affine scans.  Returns (x, steps)."""
+    x, st, _ = _run_stepped("rd_stone", a, b, c, d, dtype, (), False, 0)
+    return x, st
+
+
 def hybrid(a, b, c, d, m, inner="pcr", dtype=np.float64, log_events=False,
            log_cap=1 << 18):
     """CR+PCR (inner='pcr') or CR+RD (inner='rd') with intermediate size m
@@ -209,6 +221,8 @@ def solve(algo, a, b, c, d, m=0, dtype=np.float64):
         return pcr(a, b, c, d, dtype)[0]
     if algo == "rd":
         return rd(a, b, c, d, dtype)[0]
+    if algo == "rd_stone":
+        return rd_stone(a, b, c, d, dtype)[0]
     if algo in ("cr_pcr", "cr_rd"):
         if m <= 0:
             raise ValueError("oracle.solve needs an explicit m for the hybrids")

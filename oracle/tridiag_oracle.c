@@ -367,6 +367,103 @@ int oracle_rd_##SFX(const T* a, const T* b, const T* c, const T* d, T* x, int64_
     return oracle_hybrid_##SFX(a, b, c, d, x, n, S, 1, n, steps, log, log_cap, log_len);\
 }
 
+/* ---------------------------------------------------------------------- */
+/* Overflow-free recursive doubling in LU form (the  */
+/* paper names the overflow problem of its RD, and cites      */
+/* Stone [27] for the method).  Three Hillis-Steele scans:     */
+/*  1. pivots of A = LU: u_0 = b_0, u_i = b_i - a_i c_{i-1} / u_{i-1}, via    */
+/*     the continuant [q_i, q_{i-1}] = M_i [q_{i-1}, q_{i-2}],               */
+/*     M_i = [[b_i, -a_i c_{i-1}], [1, 0]], q_{-1} = 1, q_{-2} = 0:           */
+/*     P_i = M_i ... M_0 (later matrix on the left), u_i = P_i[0][0] /       */
+/*     P_i[1][0]; every product is rescaled by a power of two (exact) so     */
+/*     that its largest entry lies in [1, 2): no overflow, same ratios;      */
+/*  2. L y = d, l_i = a_i / u_{i-1}: affine maps y -> -l_i y + d_i composed  */
+/*     from the left (y_0 = d_0);                                           */
+/*  3. U x = y: affine maps x -> -(c_i/u_i) x + y_i/u_i composed from the    */
+/*     right (x_{n-1} = y_{n-1}/u_{n-1}).                                    */
+/* Steps: 3 log2 n scan steps + 3 setup steps + 1 evaluation.               */
+/* ---------------------------------------------------------------------- */
+#define DEFINE_STONE(T, SFX)                                                           \
+static void stone_rescale_##SFX(T* M) { /* M[4] = [[m0 m1],[m2 m3]] */                  \
+    T mx = 0;                                                                          \
+    for (int e = 0; e < 4; ++e) { T v = M[e] < 0 ? -M[e] : M[e]; if (v > mx) mx = v; } \
+    if (mx > 0 && mx == mx && mx < (T)INFINITY) {                                      \
+        int ex; frexp((double)mx, &ex);                                                \
+        for (int e = 0; e < 4; ++e) M[e] = (T)ldexp((double)M[e], 1 - ex);             \
+    }                                                                                  \
+}                                                                                      \
+int oracle_rd_stone_##SFX(const T* a, const T* b, const T* c, const T* d, T* x,        \
+                          int64_t n, int64_t S, int64_t* steps, int64_t* log,          \
+                          int64_t log_cap, int64_t* log_len) {                         \
+    if (!is_pow2(n) || n < 2 || S < 0) return -1;                                      \
+    size_t nn = (size_t)n;                                                             \
+    T* w = (T*)malloc(sizeof(T) * (4 * nn + 8 * nn + 4 * nn + 3 * nn));                \
+    if (!w) return -2;                                                                 \
+    T *A = w, *B = w + nn, *C = w + 2 * nn, *D = w + 3 * nn;                           \
+    T *Pm = w + 4 * nn, *Pm2 = Pm + 4 * nn;      /* 2x2 products (4 per eq) */        \
+    T *F = Pm2 + 4 * nn, *F2 = F + 2 * nn;       /* affine maps (alpha, beta) */       \
+    T *U = F2 + 2 * nn, *Y = U + nn;                                                   \
+    evlog_t Lg = {log, log_cap, 0};                                                    \
+    int64_t st = 0;                                                                    \
+    (void)Y;                                                                           \
+    for (int64_t s = 0; s < S; ++s) {                                                  \
+        evlog_t* L = (s == 0) ? &Lg : NULL;                                            \
+        (void)L;                                                                       \
+        T* X = x + s * n;                                                              \
+        load_sys_##SFX(a + s * n, b + s * n, c + s * n, d + s * n, n, A, B, C, D);     \
+        st = 1; /* setup of M_i */                                                     \
+        for (int64_t i = 0; i < n; ++i) {                                              \
+            T* M = Pm + 4 * i;                                                         \
+            M[0] = B[i]; M[1] = (i > 0) ? -A[i] * C[i - 1] : (T)0; M[2] = 1; M[3] = 0;  \
+        }                                                                              \
+        for (int64_t sh = 1; sh < n; sh *= 2) {                                        \
+            ++st;                                                                      \
+            memcpy(Pm2, Pm, sizeof(T) * 4 * nn);                                       \
+            for (int64_t i = sh; i < n; ++i) {                                         \
+                const T* P = Pm2 + 4 * i; const T* Q = Pm2 + 4 * (i - sh);             \
+                T* R = Pm + 4 * i;                                                     \
+                R[0] = P[0] * Q[0] + P[1] * Q[2]; R[1] = P[0] * Q[1] + P[1] * Q[3];    \
+                R[2] = P[2] * Q[0] + P[3] * Q[2]; R[3] = P[2] * Q[1] + P[3] * Q[3];    \
+                stone_rescale_##SFX(R);                                                \
+            }                                                                          \
+        }                                                                              \
+        for (int64_t i = 0; i < n; ++i) U[i] = Pm[4 * i] / Pm[4 * i + 2];              \
+        ++st; /* setup of the forward maps */                                          \
+        for (int64_t i = 0; i < n; ++i) {                                              \
+            F[2 * i] = (i > 0) ? -(A[i] / U[i - 1]) : (T)0; F[2 * i + 1] = D[i];        \
+        }                                                                              \
+        for (int64_t sh = 1; sh < n; sh *= 2) {                                        \
+            ++st;                                                                      \
+            memcpy(F2, F, sizeof(T) * 2 * nn);                                         \
+            for (int64_t i = sh; i < n; ++i) {   /* F_i o F_{i-sh} */                  \
+                F[2 * i] = F2[2 * i] * F2[2 * (i - sh)];                               \
+                F[2 * i + 1] = F2[2 * i] * F2[2 * (i - sh) + 1] + F2[2 * i + 1];       \
+            }                                                                          \
+        }                                                                              \
+        ++st; /* setup of the backward maps from y_i = F_i.beta */                     \
+        for (int64_t i = 0; i < n; ++i) {                                              \
+            T yi = F[2 * i + 1];                                                       \
+            F2[2 * i] = (i < n - 1) ? -(C[i] / U[i]) : (T)0;                           \
+            F2[2 * i + 1] = yi / U[i];                                                 \
+        }                                                                              \
+        memcpy(F, F2, sizeof(T) * 2 * nn);                                             \
+        for (int64_t sh = 1; sh < n; sh *= 2) {                                        \
+            ++st;                                                                      \
+            memcpy(F2, F, sizeof(T) * 2 * nn);                                         \
+            for (int64_t i = 0; i + sh < n; ++i) {  /* G_i o G_{i+sh} */               \
+                F[2 * i] = F2[2 * i] * F2[2 * (i + sh)];                               \
+                F[2 * i + 1] = F2[2 * i] * F2[2 * (i + sh) + 1] + F2[2 * i + 1];       \
+            }                                                                          \
+        }                                                                              \
+        ++st; /* evaluation: x_i = G_i.beta (the last map is constant) */              \
+        for (int64_t i = 0; i < n; ++i) X[i] = F[2 * i + 1];                           \
+    }                                                                                  \
+    if (steps) *steps = st;                                                            \
+    if (log_len) *log_len = Lg.len;                                                    \
+    free(w);                                                                           \
+    return 0;                                                                          \
+}
+
 #define DEFINE_ALL(T, SFX)  \
     DEFINE_THOMAS(T, SFX)   \
     DEFINE_CR_LEVELS(T, SFX) \
@@ -374,7 +471,8 @@ int oracle_rd_##SFX(const T* a, const T* b, const T* c, const T* d, T* x, int64_
     DEFINE_CR(T, SFX)       \
     DEFINE_PCR_CORE(T, SFX) \
     DEFINE_RD_CORE(T, SFX)  \
-    DEFINE_HYBRID(T, SFX)
+    DEFINE_HYBRID(T, SFX)   \
+    DEFINE_STONE(T, SFX)
 
 DEFINE_ALL(double, f64)
 DEFINE_ALL(float, f32)

@@ -1,0 +1,9 @@
+// Kernel instantiations of libtridiag.so for T = double, inner = STONE (the
+// overflow-free LU-form recursive doubling, NEXT f3).
+#include "launch.cuh"
+
+namespace tdg_host {
+template cudaError_t dispatch_t<double, tdg::kSTONE>(const void*, const void*, const void*,
+                                                const void*, void*, int64_t, int64_t, int,
+                                                cudaStream_t, int, int64_t, Layout);
+}  // namespace tdg_host

@@ -82,6 +82,8 @@ template <typename T, int R, int INNER>
 cudaError_t launch_warp(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
                         int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
   constexpr int LR = ilog2c(R);
+  if constexpr (INNER == tdg::kSTONE)  // k = 0 always: the whole system in registers
+    return launch_warp_k<T, R, INNER, (LR > 0 ? 0 : -1)>(a, b, c, d, x, n, S, 0, vec, st, nr, L);
   if (k >= LR) return launch_warp_k<T, R, INNER, -1>(a, b, c, d, x, n, S, k, vec, st, nr, L);
   switch (k) {
     case 0: return launch_warp_k<T, R, INNER, 0>(a, b, c, d, x, n, S, k, vec, st, nr, L);
@@ -186,7 +188,9 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
     }
     return cudaErrorInvalidValue;
   }
-  if constexpr (sizeof(T) == 4) {
+  if constexpr (INNER == tdg::kSTONE) {
+    return cudaErrorInvalidValue;  // n <= 32 R only (tridiag_max_n)
+  } else if constexpr (sizeof(T) == 4) {
     switch (p.W) {
       case 2: return launch_cta<T, 16, 2, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);
       case 4: return launch_cta<T, 16, 4, INNER>(a, b, c, d, x, n, S, k, vec, st, nr, L);

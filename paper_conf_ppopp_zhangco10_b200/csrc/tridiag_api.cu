@@ -202,14 +202,14 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
   // NULL pointers are legal only for an empty batch (nothing is accessed).
   if (S != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
-  if (algo < TRIDIAG_CR || algo > TRIDIAG_CR_RD) return TRIDIAG_ERR_ALGO;
+  if (algo < TRIDIAG_CR || algo > TRIDIAG_RD_STONE) return TRIDIAG_ERR_ALGO;
   if (n < 1) return TRIDIAG_ERR_N;
   const int64_t np = pad_n(n);
   if (np > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
   if (S < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
   int64_t m;
   if (algo == TRIDIAG_CR) m = 2;
-  else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD) m = np;
+  else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD || algo == TRIDIAG_RD_STONE) m = np;
   else m = switch_level == 0 ? tridiag_auto_switch_level(np, dtype, algo) : switch_level;
   if (!is_hybrid(algo) && switch_level != 0) return TRIDIAG_ERR_SWITCH_LEVEL;
   if (is_hybrid(algo)) {
@@ -235,14 +235,18 @@ int solve_device(const void* a, const void* b, const void* c, const void* d, voi
   if (S == 0) return TRIDIAG_OK;
   const int64_t n = pad_n(nr);
   const int k = ilog2_64(n / m);
-  const int inner = (algo == TRIDIAG_RD || algo == TRIDIAG_CR_RD) ? tdg::kRD : tdg::kPCR;
+  const int inner = (algo == TRIDIAG_RD || algo == TRIDIAG_CR_RD) ? tdg::kRD
+                    : algo == TRIDIAG_RD_STONE                     ? tdg::kSTONE
+                                                                   : tdg::kPCR;
   cudaError_t e;
   if (dtype == TRIDIAG_F32)
     e = inner == tdg::kPCR ? dispatch_t<float, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
-                           : dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
+        : inner == tdg::kRD ? dispatch_t<float, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
+                            : dispatch_t<float, tdg::kSTONE>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
   else
     e = inner == tdg::kPCR ? dispatch_t<double, tdg::kPCR>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
-                           : dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
+        : inner == tdg::kRD ? dispatch_t<double, tdg::kRD>(a, b, c, d, x, n, S, k, st, dtype, nr, L)
+                            : dispatch_t<double, tdg::kSTONE>(a, b, c, d, x, n, S, k, st, dtype, nr, L);
   return e == cudaSuccess ? TRIDIAG_OK : (int)e;
 }
 
@@ -288,6 +292,7 @@ int64_t tridiag_max_n(int dtype, int algo) {
     case TRIDIAG_CR_RD: return max_n_cr(dtype);
     case TRIDIAG_PCR:
     case TRIDIAG_RD: return max_inner_m(dtype);
+    case TRIDIAG_RD_STONE: return dtype == TRIDIAG_F32 ? 512 : 256;  // one warp, registers only
   }
   return 0;
 }

@@ -54,7 +54,10 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
   heads_from_next_lane<T, R>(a, b, c, d, kin, P, ls == P - 1, H);
   inlane_tail_chain<T, R>(a, b, c, d, kin, H);
   st.mark(2);
-  if constexpr (KB < 0) {
+  if constexpr (INNER == kSTONE) {
+    // overflow-free LU-form RD on the whole system (k = 0, kin = 0)
+    blocked_stone<T, R>(a, b, c, d, ls, P);
+  } else if constexpr (KB < 0) {
     d[R - 1] = lane_level_solve<T, INNER>(a[R - 1], b[R - 1], c[R - 1], d[R - 1], k - LR, ls, P);
   } else {
     // m = P * (R >> KB) > P: the intermediate system stays block-distributed
@@ -222,7 +225,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 // registers; the few spills land in the otherwise unused L1) doubles the
 // warps that hide the shuffle / MUFU latency.
 template <typename T, int R, int INNER, int KB, bool GEN>
-__global__ void __launch_bounds__(256, R >= 8 ? TDG_BLOCKED_MINB : 1)
+__global__ void __launch_bounds__(256, (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : 1)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {

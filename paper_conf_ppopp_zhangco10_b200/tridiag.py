@@ -15,7 +15,7 @@ import torch
 
 from . import build as _build
 
-ALGOS = {"cr": 0, "pcr": 1, "rd": 2, "cr_pcr": 3, "cr_rd": 4}
+ALGOS = {"cr": 0, "pcr": 1, "rd": 2, "cr_pcr": 3, "cr_rd": 4, "rd_stone": 5}
 DTYPES = {torch.float32: 0, torch.float64: 1}
 HYBRIDS = ("cr_pcr", "cr_rd")
 
@@ -173,7 +173,8 @@ def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None
     transposed views such as ``grid.T`` for the column sweep of ADI
     (tridiag_solve_batched_strided).
     x: output tensor with the same strides (may be d itself); allocated if None.
-    algo: 'cr' | 'pcr' | 'rd' | 'cr_pcr' | 'cr_rd'.
+    algo: 'cr' | 'pcr' | 'rd' | 'cr_pcr' | 'cr_rd' (the paper's five) | 'rd_stone'
+      (overflow-free LU-form recursive doubling, n <= 512 fp32 / 256 fp64).
     switch_level: intermediate size m of the hybrids (0 = tuned table).
     Enqueued asynchronously on ``stream`` (default: torch's current stream).
     """

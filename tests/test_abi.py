@@ -58,12 +58,13 @@ def test_ragged_n_is_accepted(n):
 
 def test_n_too_large():
     for dtype in (F32, F64):
-        for algo in range(5):
+        for algo in range(6):
             mx = td.max_n(dtype, algo)
-            assert mx >= 512 and (mx & (mx - 1)) == 0
+            assert mx >= 256 and (mx & (mx - 1)) == 0
             assert solve(n=2 * mx, dtype=dtype, algo=algo) == -3
             assert solve(n=mx + 1, dtype=dtype, algo=algo) == -3   # pads to 2 mx
     assert td.max_n(F32, CR_PCR) == 8192 and td.max_n(F64, CR_PCR) == 4096
+    assert td.max_n(F32, 5) == 512 and td.max_n(F64, 5) == 256   # rd_stone: one warp
     assert td.max_n(7, CR) == 0 and td.max_n(F32, 9) == 0
 
 
@@ -71,12 +72,12 @@ def test_bad_num_systems_dtype_algo():
     assert solve(S=-1) == -4
     assert solve(dtype=2) == -5
     assert solve(dtype=-1) == -5
-    assert solve(algo=5) == -6
+    assert solve(algo=6) == -6
     assert solve(algo=-1) == -6
 
 
 def test_switch_level_validation():
-    for algo in (CR, PCR, RD):
+    for algo in (CR, PCR, RD, 5):
         assert solve(algo=algo, m=4) == -7
     for algo in (CR_PCR, CR_RD):
         assert solve(algo=algo, m=3) == -7

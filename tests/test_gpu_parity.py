@@ -203,6 +203,32 @@ def test_rd_on_dd_reports_instability_not_errors():
         assert (e > 1e-4).any()
 
 
+# --------------------------------------------------------------------------- LU-form RD (NEXT f3)
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_rd_stone_meets_the_dd_gates(dtype):
+    """The overflow-free LU-form recursive doubling passes G1/G2/G3 on the
+    dominant families where the paper's RD fails (R24)."""
+    for n in n_list(dtype, "rd_stone"):
+        for fam, kw in [("dd", {}), ("km", {"E": 1.0}), ("km", {"E": 100.0})]:
+            a, b, c, d = gen(fam, RAGGED_S, n, dtype, seed=n, **kw)
+            e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "rd_stone"))
+            assert e.max() <= TOL[dtype], (fam, n, e.max())
+        a, b, c, d = gen("poi", 64, n, dtype, seed=n)
+        e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "rd_stone"))
+        assert e.max() <= (1e-3 if dtype == torch.float32 else 1e-10), (n, e.max())
+    # same method as the oracle's rd_stone: within 10x of its error
+    a, b, c, d = gen("dd", 32, 256, dtype)
+    ha, hb, hc, hd = host(a, b, c, d)
+    e_o = oracle.normwise_error(oracle.rd_stone(ha, hb, hc, hd, dtype=np.float32 if dtype == torch.float32 else np.float64)[0],
+                                oracle.thomas(ha, hb, hc, hd)).max()
+    e_g = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "rd_stone")).max()
+    assert e_g <= 10 * max(e_o, 1e-15)
+    # ragged n and columns take the same kernel
+    for n in [5, 100]:
+        a, b, c, d = gen("dd", 40, n, dtype, seed=n)
+        assert err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, "rd_stone")).max() <= TOL[dtype]
+
+
 # --------------------------------------------------------------------------- ragged n (NEXT f2)
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
 def test_ragged_n(dtype):

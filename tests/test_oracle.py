@@ -375,3 +375,30 @@ def test_residual_metric_definition():
     A = dense(a[0], b[0], c[0])
     assert oracle.residual_inf(a, b, c, d, x)[0] == pytest.approx(np.max(np.abs(A @ x[0] - d[0])), abs=1e-15)
     assert np.max(scipy.linalg.norm(A @ x[0] - d[0], np.inf)) <= 1e-14
+
+
+# ----------------------------------------------------------------------------- RD in LU form (NEXT f3)
+@pytest.mark.parametrize("family,kw", [("dd", {}), ("km", {"E": 1.0}), ("km", {"E": 100.0}), ("poi", {})])
+@pytest.mark.parametrize("n", [2, 4, 16, 64, 512, 4096])
+def test_rd_stone_matches_lapack(family, kw, n):
+    """The overflow-free LU-form RD solves the dominant families where the
+    paper's RD overflows: vs LAPACK dgtsv."""
+    a, b, c, d = gen(family, 3, n, seed=31 + n, **kw)
+    x, st = oracle.rd_stone(a, b, c, d)
+    tol = 1e-13 if family != "poi" else 1e-10
+    assert oracle.normwise_error(x, gtsv(a, b, c, d)).max() <= tol
+    assert st == 3 * int(math.log2(n)) + 4     # 3 scans + 3 setups + evaluation
+
+
+def test_rd_stone_dense_small_and_no_overflow():
+    for n in [2, 4, 8, 16]:
+        a, b, c, d = gen("cv", 4, n, seed=n)
+        ref = np.stack([np.linalg.solve(dense(a[s], b[s], c[s]), d[s]) for s in range(4)])
+        assert oracle.normwise_error(oracle.rd_stone(a, b, c, d)[0], ref).max() <= 1e-12
+    # (1, 4, 1) rows: the paper's RD overflows in fp32 beyond n = 64; this form does not
+    n = 8192
+    a = np.ones((2, n), np.float32); c = np.ones((2, n), np.float32); b = 4 * np.ones((2, n), np.float32)
+    d = np.random.default_rng(0).uniform(-1, 1, (2, n)).astype(np.float32)
+    x32, _ = oracle.rd_stone(a, b, c, d, dtype=np.float32)
+    assert np.all(np.isfinite(x32))
+    assert oracle.normwise_error(x32, oracle.thomas(a, b, c, d)).max() <= 1e-5
