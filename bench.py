@@ -371,7 +371,7 @@ def main():
         line["e2e"] = {"value": total * e2e_steps / e2e_t, "unit": UNIT,
                        "h2d_bytes_per_step": 4 * n * T * S, "d2h_bytes_per_step": n * T * S,
                        "how": f"tridiag_solve_batched_host on pinned host buffers, {chunk}-system "
-                              f"chunks pipelined over 2 streams, {e2e_steps} steps, wall clock "
+                              f"chunks pipelined over 3 streams, {e2e_steps} steps, wall clock "
                               f"around the blocking call, max over ranks"}
         del ws, ha, hb, hc, hd, hx
         # --- every algorithm on the same workload (RD family on the RD-stable POI input)

@@ -137,8 +137,8 @@ int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, c
  * "with transfer" case).  a, b, c, d, x are host pointers
  * (pinned memory gives full-speed asynchronous copies; pageable memory works
  * but serialises).  The batch is split into chunks that are pipelined over
- * two CUDA streams: the host-to-device copy of chunk j+1 and the
- * device-to-host copy of chunk j-1 overlap the solve of chunk j.
+ * three CUDA streams / buffers: host-to-device copies of the next chunks and
+ * the device-to-host copy of earlier ones overlap the solve of chunk j.
  *
  * workspace        device buffer owned by the caller, at least
  *                  tridiag_host_workspace_bytes(n, dtype, chunk_systems) bytes.

@@ -329,10 +329,15 @@ int tridiag_solve_batched(const void* a, const void* b, const void* c, const voi
                                        switch_level, stream);
 }
 
+// Host pipeline depth: three chunk buffers on three streams, so the
+// host-to-device engine can run ahead of a device-to-host copy that still
+// occupies the previous buffer.
+constexpr int kHostBufs = 3;
+
 size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems) {
   if (n < 1 || chunk_systems < 0 || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return 0;
   if (chunk_systems == 0) chunk_systems = std::max<int64_t>(1, (int64_t(16) << 20) / (4 * n * (int64_t)elem_size(dtype)));
-  return (size_t)2 * 4 * (size_t)chunk_systems * (size_t)n * elem_size(dtype);
+  return (size_t)kHostBufs * 4 * (size_t)chunk_systems * (size_t)n * elem_size(dtype);
 }
 
 int tridiag_solve_batched_host(const void* a, const void* b, const void* c, const void* d, void* x,
@@ -353,11 +358,12 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
 
   const size_t T = elem_size(dtype);
   const size_t arr = (size_t)chunk_systems * (size_t)n * T;  // one array of one chunk
-  cudaStream_t st[2];
-  if (cudaStreamCreateWithFlags(&st[0], cudaStreamNonBlocking) != cudaSuccess) return (int)cudaGetLastError();
-  if (cudaStreamCreateWithFlags(&st[1], cudaStreamNonBlocking) != cudaSuccess) {
-    cudaStreamDestroy(st[0]);
-    return (int)cudaGetLastError();
+  cudaStream_t st[kHostBufs];
+  for (int i = 0; i < kHostBufs; ++i) {
+    if (cudaStreamCreateWithFlags(&st[i], cudaStreamNonBlocking) != cudaSuccess) {
+      for (int j = 0; j < i; ++j) cudaStreamDestroy(st[j]);
+      return (int)cudaGetLastError();
+    }
   }
   int rc = TRIDIAG_OK;
   int launches = 0;
@@ -368,8 +374,8 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
     const int64_t cnt = std::min<int64_t>(chunk_systems, num_systems - s0);
     const size_t bytes = (size_t)cnt * (size_t)n * T;
     const size_t off = (size_t)s0 * (size_t)n * T;
-    cudaStream_t s = st[j & 1];
-    char* buf = static_cast<char*>(workspace) + (size_t)(j & 1) * 4 * arr;
+    cudaStream_t s = st[j % kHostBufs];
+    char* buf = static_cast<char*>(workspace) + (size_t)(j % kHostBufs) * 4 * arr;
     for (int q = 0; q < 4; ++q) {
       cudaError_t e = cudaMemcpyAsync(buf + q * arr, hp[q] + off, bytes, cudaMemcpyHostToDevice, s);
       if (e != cudaSuccess) { rc = (int)e; break; }
@@ -383,12 +389,11 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
     cudaError_t e = cudaMemcpyAsync(hx + off, buf + 3 * arr, bytes, cudaMemcpyDeviceToHost, s);
     if (e != cudaSuccess) rc = (int)e;
   }
-  cudaError_t e0 = cudaStreamSynchronize(st[0]);
-  cudaError_t e1 = cudaStreamSynchronize(st[1]);
-  if (rc == TRIDIAG_OK && e0 != cudaSuccess) rc = (int)e0;
-  if (rc == TRIDIAG_OK && e1 != cudaSuccess) rc = (int)e1;
-  cudaStreamDestroy(st[0]);
-  cudaStreamDestroy(st[1]);
+  for (int i = 0; i < kHostBufs; ++i) {
+    const cudaError_t e = cudaStreamSynchronize(st[i]);
+    if (rc == TRIDIAG_OK && e != cudaSuccess) rc = (int)e;
+    cudaStreamDestroy(st[i]);
+  }
   g_last_launches = launches;
   return rc;
 }

@@ -124,7 +124,7 @@ def test_python_errors_are_loud():
 
 
 def test_host_workspace_size():
-    assert td.host_workspace_bytes(512, F32, 1000) == 2 * 4 * 1000 * 512 * 4
+    assert td.host_workspace_bytes(512, F32, 1000) == 3 * 4 * 1000 * 512 * 4
     assert td.host_workspace_bytes(512, F64, 0) > 0
     L = td.load()
     # workspace too small -> -9 before any CUDA call
