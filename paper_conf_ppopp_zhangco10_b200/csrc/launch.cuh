@@ -171,7 +171,10 @@ cudaError_t dispatch_t(const void* a_, const void* b_, const void* c_, const voi
   const T* c = static_cast<const T*>(c_);
   const T* d = static_cast<const T*>(d_);
   T* x = static_cast<T*>(x_);
-  const Plan p = plan_for(dtype, n, S);
+  // The RD-family inners use a work-efficient block scan whose association
+  // depends on R, so they always take the HBM-scale plan: results stay
+  // bitwise independent of the batch size (R22).
+  const Plan p = plan_for(dtype, n, INNER == tdg::kPCR ? S : -1);
   const size_t tile = std::min<size_t>(32, (size_t)p.R * sizeof(T));
   auto al = [tile](const void* q) { return (reinterpret_cast<uintptr_t>(q) % tile) == 0; };
   const bool vec = nr == n && L.es == 1 && ((uint64_t)L.ss * sizeof(T)) % tile == 0 && al(a) &&
