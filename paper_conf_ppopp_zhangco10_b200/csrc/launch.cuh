@@ -126,7 +126,22 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
   const size_t smem = tdg::cta_tma_smem_bytes<T>(R, W, INNER, k);
   int dev = 0;
   cudaGetDevice(&dev);
-  auto kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER>;
+  constexpr int LR = ilog2c(R);
+  auto kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, -1>;
+  // RD with k <= log2 R (one survivor per lane at k = log2 R): blocked CTA scan
+  if (k < LR || (INNER == tdg::kRD && k == LR)) {
+    if constexpr (INNER != tdg::kRD) {
+      return cudaSuccess;
+    } else {
+      switch (k) {
+        case 0: kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, 0>; break;
+        case 1: kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, (LR > 1 ? 1 : 0)>; break;
+        case 2: kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, (LR > 2 ? 2 : 0)>; break;
+        case 3: kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, (LR > 3 ? 3 : 0)>; break;
+        default: kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, LR>; break;
+      }
+    }
+  }
   const int occ = occupancy(dev, kern, W * 32, smem);
   if (occ <= 0) return cudaSuccess;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
@@ -139,7 +154,8 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
-  if (vec && nr == n && L.es == 1 && L.ss == n && k >= ilog2c(R) && tma_mode()) {
+  if (vec && nr == n && L.es == 1 && L.ss == n && (k >= ilog2c(R) || INNER == tdg::kRD) &&
+      tma_mode()) {
     bool used = false;
     const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
     if (used || e != cudaSuccess) return e;
@@ -148,8 +164,22 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   const size_t smem = tdg::cta_smem_bytes<T>(R, W, INNER, k, staged);
   int dev = 0;
   cudaGetDevice(&dev);
-  auto kern = k < ilog2c(R) ? tdg::tdg_cta_kernel<T, R, W, INNER, true>
-                             : tdg::tdg_cta_kernel<T, R, W, INNER, false>;
+  constexpr int LR = ilog2c(R);
+  // RD with k < log2 R: register-blocked CTA scan compiled for that k
+  auto kern = tdg::tdg_cta_kernel<T, R, W, INNER, -1>;
+  if (k < LR || (INNER == tdg::kRD && k == LR)) {
+    if constexpr (INNER != tdg::kRD) {
+      kern = tdg::tdg_cta_kernel<T, R, W, INNER, -2>;
+    } else {
+      switch (k) {
+        case 0: kern = tdg::tdg_cta_kernel<T, R, W, INNER, 0>; break;
+        case 1: kern = tdg::tdg_cta_kernel<T, R, W, INNER, (LR > 1 ? 1 : 0)>; break;
+        case 2: kern = tdg::tdg_cta_kernel<T, R, W, INNER, (LR > 2 ? 2 : 0)>; break;
+        case 3: kern = tdg::tdg_cta_kernel<T, R, W, INNER, (LR > 3 ? 3 : 0)>; break;
+        default: kern = tdg::tdg_cta_kernel<T, R, W, INNER, LR>; break;
+      }
+    }
+  }
   const int occ = occupancy(dev, kern, W * 32, smem);
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));

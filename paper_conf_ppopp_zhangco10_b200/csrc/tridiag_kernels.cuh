@@ -396,7 +396,121 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
   return xprev;
 }
 
-template <typename T, int R, int W, int INNER, bool SMEM>
+// RD on the register-blocked m-system of a whole CTA (P = 32 W lanes, Q =
+// R >> K survivors per lane): in-lane sequential scan, Hillis-Steele over the
+// 32 lane aggregates of each warp (shuffles), one more over the W warp
+// aggregates (shared memory, warp 0), fix-up composes, evaluation (R25).
+// Returns x of the previous lane's tail for the in-lane back-substitution;
+// d[t_u] <- x of the survivors.
+template <typename T, int R, int W, int K>
+__device__ __forceinline__ T cta_blocked_rd(T (&a)[R], T (&b)[R], T (&c)[R], T (&d)[R], T* sm) {
+  constexpr int Q = R >> K;
+  constexpr int P = 32 * W;
+  const int ls = threadIdx.x;
+  const int lane = ls & 31;
+  const int warp = ls >> 5;
+  const int m = P * Q;
+  T* wagg = sm;              // [W][6] warp aggregates -> exclusive warp prefixes
+  T* tail = sm + 6 * W;      // [W][2] C[0][0], C[0][2] of every warp's last element
+  T* misc = tail + 2 * W;    // [0..1] last element's C (x0), [2 + w] last x of warp w
+  T M[Q][6];
+#pragma unroll
+  for (int u = 0; u < Q; ++u) {
+    const int t = Blocked<T, R, K>::t(u);
+    const int g = ls * Q + u;
+    rd_setup6(a[t], b[t], c[t], d[t], g == 0, g == m - 1, M[u]);
+  }
+  auto op = [](T (&p)[6], const T (&q)[6]) { mat_compose(p, q); };
+#pragma unroll
+  for (int u = 1; u < Q; ++u) op(M[u], M[u - 1]);
+  T agg[6];
+#pragma unroll
+  for (int e = 0; e < 6; ++e) agg[e] = M[Q - 1][e];
+#pragma unroll
+  for (int s = 1; s < 32; s <<= 1) {
+    T F[6];
+#pragma unroll
+    for (int e = 0; e < 6; ++e) F[e] = shup(agg[e], s, 32);
+    if (lane >= s) op(agg, F);
+  }
+  T lex[6];  // exclusive prefix within the warp
+#pragma unroll
+  for (int e = 0; e < 6; ++e) lex[e] = shup(agg[e], 1, 32);
+  if (lane == 31) {
+#pragma unroll
+    for (int e = 0; e < 6; ++e) wagg[warp * 6 + e] = agg[e];
+  }
+  __syncthreads();
+  if (warp == 0) {
+    T wv[6];
+#pragma unroll
+    for (int e = 0; e < 6; ++e) wv[e] = lane < W ? wagg[lane * 6 + e] : T(0);
+#pragma unroll
+    for (int s = 1; s < 32; s <<= 1) {
+      if (s < W) {
+        T F[6];
+#pragma unroll
+        for (int e = 0; e < 6; ++e) F[e] = shup(wv[e], s, 32);
+        if (lane >= s) op(wv, F);
+      }
+    }
+    T wx[6];
+#pragma unroll
+    for (int e = 0; e < 6; ++e) wx[e] = shup(wv[e], 1, 32);
+    __syncwarp();
+    if (lane < W) {
+#pragma unroll
+      for (int e = 0; e < 6; ++e) wagg[lane * 6 + e] = wx[e];
+    }
+  }
+  __syncthreads();
+  // prefix of everything before this lane = (earlier lanes of the warp) o (earlier warps)
+  if (ls > 0) {
+    T ex[6];
+    if (warp > 0) {
+      T wx[6];
+#pragma unroll
+      for (int e = 0; e < 6; ++e) wx[e] = wagg[warp * 6 + e];
+      if (lane > 0) {
+#pragma unroll
+        for (int e = 0; e < 6; ++e) ex[e] = lex[e];
+        op(ex, wx);
+      } else {
+#pragma unroll
+        for (int e = 0; e < 6; ++e) ex[e] = wx[e];
+      }
+    } else {
+#pragma unroll
+      for (int e = 0; e < 6; ++e) ex[e] = lex[e];
+    }
+#pragma unroll
+    for (int u = 0; u < Q; ++u) op(M[u], ex);
+  }
+  // evaluation: x_0 from the last element, x_g from C_{g-1}
+  if (ls == P - 1) { misc[0] = M[Q - 1][0]; misc[1] = M[Q - 1][2]; }
+  if (lane == 31) { tail[warp * 2] = M[Q - 1][0]; tail[warp * 2 + 1] = M[Q - 1][2]; }
+  __syncthreads();
+  const T x0 = rd_x0(misc[0], misc[1]);
+  T p00 = shup(M[Q - 1][0], 1, 32), p02 = shup(M[Q - 1][2], 1, 32);
+  if (lane == 0 && warp > 0) { p00 = tail[(warp - 1) * 2]; p02 = tail[(warp - 1) * 2 + 1]; }
+#pragma unroll
+  for (int u = Q - 1; u >= 0; --u) {
+    const int t = Blocked<T, R, K>::t(u);
+    if (u > 0) d[t] = rd_eval(M[u - 1][0], M[u - 1][2], x0);
+    else d[t] = (ls == 0) ? x0 : rd_eval(p00, p02, x0);
+  }
+  // x of the previous lane's tail (its last survivor) for the back-substitution
+  if (lane == 31) misc[2 + warp] = d[R - 1];
+  __syncthreads();
+  T xprev = shup(d[R - 1], 1, 32);
+  if (lane == 0) xprev = warp > 0 ? misc[2 + warp - 1] : T(0);
+  return xprev;
+}
+
+// KB = -1: register path (k >= log2 R).  KB = -2: shared-memory inner for
+// k < log2 R (runtime k; PCR).  KB >= 0: k = KB < log2 R with the register-
+// blocked inner across the CTA (RD: cta_blocked_rd).
+template <typename T, int R, int W, int INNER, int KB>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                const T* d, T* x, int n, long long S, int k, int vec, int pf, int n_real,
@@ -411,7 +525,8 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
   const int ls = threadIdx.x;
   const int lane = ls & 31;
   const int warp = ls >> 5;
-  const int kin = SMEM ? (k < LR ? k : LR) : LR;
+  constexpr bool SMEM = KB != -1;
+  const int kin = KB >= 0 ? KB : SMEM ? (k < LR ? k : LR) : LR;
 
   for (long long sys = blockIdx.x; sys < S; sys += gridDim.x) {
     if (pf && lane < 4 && sys + gridDim.x < S) {
@@ -474,6 +589,8 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
     T xprev;
     if constexpr (!SMEM) {
       xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
+    } else if constexpr (KB >= 0 && INNER == kRD) {
+      xprev = cta_blocked_rd<T, R, W, (KB >= 0 ? KB : 0)>(ra, rb, rc, rd, work);
     } else {
       // ---- m = P * q > P: shared-memory inner on the whole CTA ----
       const int q = R >> k;
@@ -528,7 +645,7 @@ inline size_t cta_smem_bytes_core(int R, int W, int inner, int k) {
   const int LR = ilog2c(R);
   const int LRH = LR > 0 ? LR : 1;
   int64_t e = (int64_t)W * LRH * 4;
-  if (k >= LR) {
+  if (k > LR || (k == LR && inner != kRD)) {
     const int kr = k - LR;
     const int kl = kr < 5 ? kr : 5;
     const int64_t msurv = (int64_t)W * (32 >> kl);
@@ -536,7 +653,8 @@ inline size_t cta_smem_bytes_core(int R, int W, int inner, int k) {
     if (msurv > 32) e += inner_region_elems(inner, msurv);
   } else {
     const int64_t m = (int64_t)P * (R >> k);
-    e += inner_region_elems(inner, m);
+    // RD: cta_blocked_rd's warp aggregates, tails and broadcasts only
+    e += inner == kRD ? 9LL * W + 2 : inner_region_elems(inner, m);
   }
   return (size_t)e * sizeof(T);
 }

@@ -74,7 +74,9 @@ __host__ __device__ constexpr uint32_t tma_stage_bytes(int R, int W) {
   return (uint32_t)(((4u * 32u * W * R * sizeof(T)) + 1023u) & ~1023u);
 }
 
-template <typename T, int R, int W, int INNER>
+// KB = -1: k >= log2 R (register path); KB >= 0: RD inner with k = KB
+// (cta_blocked_rd).
+template <typename T, int R, int W, int INNER, int KB>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
@@ -122,11 +124,17 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     if (ls == P - 1) rc[R - 1] = T(0);
     const long long next = sys + gridDim.x;
     // every thread has read the stage once the heads barrier is passed
-    cta_inlane_forward<T, R, W>(ra, rb, rc, rd, LR, heads, [&] {
+    constexpr int KIN = KB >= 0 ? KB : LR;
+    cta_inlane_forward<T, R, W>(ra, rb, rc, rd, KIN, heads, [&] {
       if (ls == 0 && next < S) issue(next);
     });
-    const T xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
-    inlane_backward<T, R>(ra, rb, rc, rd, LR, xprev);
+    T xprev;
+    if constexpr (KB >= 0) {
+      xprev = cta_blocked_rd<T, R, W, (KB >= 0 ? KB : 0)>(ra, rb, rc, rd, heads + W * (LR > 0 ? LR : 1) * 4);
+    } else {
+      xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
+    }
+    inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
     store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
     __syncthreads();  // heads / survivor regions are reused by the next system
   }

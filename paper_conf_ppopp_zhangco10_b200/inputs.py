@@ -28,13 +28,19 @@ so these are the readings R19 of DESIGN.md):
 * ``poi``  a = c = -1, b = 2; d ~ U(-1,1)   (weakly dominant, RD-stable)
 * ``poi1`` a = c = -1, b = 2, d = 1: closed form x_i = (i+1)(n-i)/2.
 * ``cv``   a_i, b_i, c_i ~ U(0.9,1.1); d ~ U(-1,1)  ("close values in all rows")
+* ``rdw``  a_i ~ U(-0.01,0.01), b_i, c_i ~ U(0.99,1.01); d ~ U(-1,1).  Not a
+           paper workload: a test family on which RD's forward recurrence
+           x_{i+1} = (d_i - a_i x_{i-1} - b_i x_i) / c_i (the B_i of P:L398-401) neither
+           overflows nor amplifies error at large n (characteristic roots
+           ~ -b/c and ~ -a/b), so RD / CR+RD kernels can be held to the
+           accuracy gates at the CTA sizes (n > 32 R).
 """
 from __future__ import annotations
 
 import torch
 
 M32 = 0xFFFFFFFF
-FAMILIES = ("dd", "km", "poi", "poi1", "cv")
+FAMILIES = ("dd", "km", "poi", "poi1", "cv", "rdw")
 DEFAULT_SEED = 20100109  # SURVEY.md 8(d): seed = 20100109 + config index
 
 
@@ -119,6 +125,11 @@ def generate(family: str, S: int, n: int, dtype=torch.float32, seed: int = DEFAU
             d = 2.0 * uniform(g, seed, 4) - 1.0
         else:
             d = torch.ones(g.shape, dtype=f64, device=device)
+    elif family == "rdw":
+        a = 0.02 * uniform(g, seed, 0) - 0.01
+        b = 0.99 + 0.02 * uniform(g, seed, 2)
+        c = 0.99 + 0.02 * uniform(g, seed, 1)
+        d = 2.0 * uniform(g, seed, 4) - 1.0
     else:  # cv
         a = 0.9 + 0.2 * uniform(g, seed, 0)
         b = 0.9 + 0.2 * uniform(g, seed, 2)

@@ -6,6 +6,7 @@ upcast of the T-typed inputs (reading R18), max over systems:
   G1/G2  CR, PCR, CR+PCR (every m)  DD        fp32 1e-4 / fp64 1e-10
   G3     same                        KM(1), KM(100)
   G4     RD, CR+RD                   POI       fp64 1e-10 (n <= 512)
+  G4'    RD, CR+RD (every n, m)       rdw       fp32 1e-4 / fp64 1e-10
   G5     RD                          POI       fp32 1e-4  (n <= 32)
   G5'    CR+RD                       POI       fp32 1e-4  (n <= 64)
   G6     POI, d = 1 closed form: exact for CR, RD, CR+RD; PCR family <= 4 ulp
@@ -105,6 +106,19 @@ def test_rd_family_poisson_fp64(algo):
             x = gpu_solve(a, b, c, d, algo, m)
             e = err_vs_oracle(a, b, c, d, x)
             assert e.max() <= 1e-10, (algo, n, m, e.max())
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_rd_family_rdw_every_size_and_m(dtype):
+    """G4' on the RD-stable rdw family: RD and CR+RD at every n up to max_n and
+    every m, covering the warp kernels and the CTA kernels (register-blocked
+    CTA scan for m > 32 lanes, k = 0..log2 R - 1; TMA-fed when aligned)."""
+    for algo in ("rd", "cr_rd"):
+        for n in n_list(dtype, algo):
+            a, b, c, d = gen("rdw", S_for(n), n, dtype, seed=n)
+            for m in (m_list(n, dtype, algo) if algo == "cr_rd" else [0]):
+                e = err_vs_oracle(a, b, c, d, gpu_solve(a, b, c, d, algo, m))
+                assert e.max() <= TOL[dtype], (algo, n, m, e.max())
 
 
 def test_rd_poisson_fp32():

@@ -34,6 +34,25 @@ def test_families_have_their_structure():
     a, b, c, d = [t.numpy() for t in inputs.generate("cv", 3, n, torch.float64)]
     for v in (a, b, c):
         assert np.all((v >= 0.9) & (v < 1.1))
+    a, b, c, d = [t.numpy() for t in inputs.generate("rdw", 3, n, torch.float64)]
+    assert np.all(np.abs(a) <= 0.01)
+    for v in (b, c):
+        assert np.all((v >= 0.99) & (v < 1.01))
+
+
+def test_rdw_is_rd_stable_in_the_oracle():
+    """The rdw family's premise: the oracle's RD (fp64 and fp32) stays close
+    to Thomas at n = 4096, where RD on DD / KM overflows in fp32."""
+    import oracle
+    a, b, c, d = [t.numpy() for t in inputs.generate("rdw", 4, 4096, torch.float64)]
+    ref = oracle.thomas(a, b, c, d)
+    x64, _, _ = oracle.rd(a, b, c, d)
+    assert oracle.normwise_error(x64, ref).max() < 1e-11
+    a, b, c, d = [t.numpy() for t in inputs.generate("rdw", 4, 4096, torch.float32)]
+    ref = oracle.thomas(a, b, c, d)
+    x32, _, _ = oracle.rd(a, b, c, d, dtype=np.float32)
+    assert np.isfinite(x32).all()
+    assert oracle.normwise_error(x32, ref).max() < 1e-4
 
 
 def test_poison_corners_and_rounding():
