@@ -59,7 +59,8 @@ enum {
     TRIDIAG_ERR_SWITCH_LEVEL = -7, /* invalid switch_level for this algo / n / dtype */
     TRIDIAG_ERR_OVERLAP = -8,      /* x overlaps an input other than exactly x == d  */
     TRIDIAG_ERR_WORKSPACE = -9,    /* host entry point: workspace too small / NULL   */
-    TRIDIAG_ERR_STRIDE = -10       /* strided entry point: invalid strides           */
+    TRIDIAG_ERR_STRIDE = -10,      /* strided entry point: invalid strides           */
+    TRIDIAG_ERR_BOTTOM_N = -11     /* large-n entry point: invalid bottom_n          */
 };
 
 /*
@@ -151,6 +152,54 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
                                int switch_level, void* workspace, size_t workspace_bytes,
                                int64_t chunk_systems);
 size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems);
+
+/*
+ * tridiag_solve_batched_large -- systems larger than tridiag_max_n (SURVEY.md
+ * 8(f) NEXT f2; "accelerate larger systems with several first steps (as in
+ * CR) that reduce the system to fit into shared memory").
+ *
+ * Same arguments, semantics, layout (contiguous, system stride n) and errors
+ * as tridiag_solve_batched, for CR, CR+PCR and CR+RD with
+ * n_pad <= tridiag_max_n_large(dtype, algo) (2^30).  PCR, RD and RD_STONE
+ * have no CR levels to reduce with: for them (and for any n_pad <= bottom_n)
+ * this is exactly tridiag_solve_batched.
+ *
+ * Method: passes of log2 R CR levels (R = 16 fp32 / 8 fp64 equations per
+ * lane; chunks of tridiag_large_chunk(dtype) equations per CTA) write the
+ * surviving n / R equations of every system to the workspace, until the
+ * system has at most bottom_n equations; the on-chip kernels solve it (CR,
+ * or the hybrid with intermediate size m); expansion passes recompute each
+ * level's forward steps from its input and back-substitute.  Every equation
+ * update is the same correctly rounded operation sequence as in the on-chip
+ * kernels, so CR and CR+PCR results are bitwise identical to
+ * tridiag_solve_batched wherever both apply.  HBM traffic is about
+ * 10 n T bytes per system (each level read twice) against 5 n T on chip.
+ *
+ * switch_level  hybrids: 0 = the tuned m of the size the passes reduce to;
+ *             else a power of two m with 2 <= m <= tridiag_max_switch_level
+ *             at that size (m caps the CR levels: the passes stop at m).
+ * bottom_n    largest system solved on chip; 0 = tridiag_max_n(dtype, CR),
+ *             else a power of two in [tridiag_large_chunk(dtype) / 2,
+ *             tridiag_max_n(dtype, CR)] (TRIDIAG_ERR_BOTTOM_N otherwise).
+ * workspace   device buffer owned by the caller, >= tridiag_large_workspace_bytes
+ *             bytes (256-byte aligned for the vector path; NULL allowed when
+ *             that is 0).  Holds the reduced systems (4 arrays per level, the
+ *             deepest one solved in place) and the chunk-boundary head
+ *             equations; about 4 S n T / (R - 1) bytes.
+ * Asynchronous on `stream` like tridiag_solve_batched; x == d allowed.
+ */
+int tridiag_solve_batched_large(const void* a, const void* b, const void* c, const void* d,
+                                void* x, int64_t n, int64_t num_systems, int dtype, int algo,
+                                int switch_level, int64_t bottom_n, void* workspace,
+                                int64_t workspace_bytes, tridiag_stream_t stream);
+/* Workspace bytes tridiag_solve_batched_large needs (0 when n fits on chip);
+ * -1 for invalid arguments. */
+int64_t tridiag_large_workspace_bytes(int64_t n, int64_t num_systems, int dtype, int algo,
+                                      int switch_level, int64_t bottom_n);
+/* Largest n of tridiag_solve_batched_large for (dtype, algo); 0 if invalid. */
+int64_t tridiag_max_n_large(int dtype, int algo);
+/* Equations per reduction chunk (one CTA) of the large-n passes. */
+int64_t tridiag_large_chunk(int dtype);
 
 /* Human-readable text of a status code (static storage, never NULL). */
 const char* tridiag_status_string(int status);

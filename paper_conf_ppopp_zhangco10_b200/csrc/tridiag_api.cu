@@ -10,6 +10,7 @@
 #include <map>
 #include <mutex>
 #include <tuple>
+#include <vector>
 
 #include "host_common.h"
 #include "tridiag_device.cuh"  // tdg::kPCR / kRD, ilog2c
@@ -200,21 +201,29 @@ bool overlaps(const void* p, const void* q, size_t bytes) {
 // On success *m_out is the resolved intermediate size m (n for PCR/RD, 2 for CR).
 int validate(const void* a, const void* b, const void* c, const void* d, const void* x,
              int64_t n, int64_t S, int dtype, int algo, int switch_level, int64_t* m_out,
-             int64_t es, int64_t ss) {
+             int64_t es, int64_t ss, bool large = false) {
   // NULL pointers are legal only for an empty batch (nothing is accessed).
   if (S != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
   if (algo < TRIDIAG_CR || algo > TRIDIAG_RD_STONE) return TRIDIAG_ERR_ALGO;
   if (n < 1) return TRIDIAG_ERR_N;
   const int64_t np = pad_n(n);
-  if (np > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
+  if (np > (large ? tridiag_max_n_large(dtype, algo) : tridiag_max_n(dtype, algo)))
+    return TRIDIAG_ERR_N_TOO_LARGE;
   if (S < 0) return TRIDIAG_ERR_NUM_SYSTEMS;
   int64_t m;
   if (algo == TRIDIAG_CR) m = 2;
   else if (algo == TRIDIAG_PCR || algo == TRIDIAG_RD || algo == TRIDIAG_RD_STONE) m = np;
   else m = switch_level == 0 ? tridiag_auto_switch_level(np, dtype, algo) : switch_level;
   if (!is_hybrid(algo) && switch_level != 0) return TRIDIAG_ERR_SWITCH_LEVEL;
-  if (is_hybrid(algo)) {
+  if (is_hybrid(algo) && large) {
+    // resolved against the level plan by solve_large
+    if (switch_level < 0 || (switch_level != 0 && (switch_level < 2 || !is_pow2(switch_level) ||
+                                                   switch_level > np ||
+                                                   switch_level > max_inner_m(dtype))))
+      return TRIDIAG_ERR_SWITCH_LEVEL;
+    m = switch_level;
+  } else if (is_hybrid(algo)) {
     if (switch_level < 0 || m < 2 || !is_pow2(m) || m > np ||
         m > tridiag_max_switch_level(dtype, algo, np))
       return TRIDIAG_ERR_SWITCH_LEVEL;
@@ -252,6 +261,144 @@ int solve_device(const void* a, const void* b, const void* c, const void* d, voi
   return e == cudaSuccess ? TRIDIAG_OK : (int)e;
 }
 
+// ---------------------------------------------------------------------------
+// Large n (NEXT f2): reduction passes of log2 R CR levels each
+// until the system fits the on-chip kernels (n <= bottom_n), the on-chip
+// solve of the reduced system, then the expansion passes in reverse.
+// ---------------------------------------------------------------------------
+struct LargeLevel {
+  int64_t n;  // padded size of this level's system
+  int kin;    // CR levels applied by its pass
+};
+int large_R(int dtype) { return dtype == TRIDIAG_F64 ? 8 : 16; }
+int64_t large_chunk_n(int dtype) {
+  return dtype == TRIDIAG_F64 ? large_chunk<double>() : large_chunk<float>();
+}
+size_t align256(size_t v) { return (v + 255) & ~size_t(255); }
+
+// Level plan for a padded size np and intermediate size m (2 for CR); false
+// if bottom_n is not a valid stopping size for this dtype.
+bool large_plan(int64_t np, int dtype, int64_t m, int64_t bottom_n, std::vector<LargeLevel>* lv,
+                int64_t* n_last) {
+  const int LR = ilog2_64(large_R(dtype));
+  const int64_t CH = large_chunk_n(dtype);
+  lv->clear();
+  int64_t cur = np;
+  while (cur > bottom_n) {
+    const int kin = std::min(LR, ilog2_64(cur / m));
+    if (kin < 1 || cur % CH != 0) return false;
+    lv->push_back({cur, kin});
+    cur >>= kin;
+  }
+  *n_last = cur;
+  return true;
+}
+
+int64_t resolve_bottom_n(int dtype, int64_t bottom_n) {
+  if (bottom_n == 0) return max_n_cr(dtype);
+  if (!is_pow2(bottom_n) || bottom_n < large_chunk_n(dtype) / 2 || bottom_n > max_n_cr(dtype)) return -1;
+  return bottom_n;
+}
+
+// m of a large solve: CR 2, PCR / RD n; hybrids the caller's m or the auto
+// table at the size the passes reduce to.  -1 if invalid.
+int64_t large_m(int64_t np, int dtype, int algo, int64_t m_req, int64_t bottom_n) {
+  if (algo == TRIDIAG_CR) return 2;
+  if (!is_hybrid(algo)) return np <= bottom_n ? np : -1;
+  std::vector<LargeLevel> lv;
+  int64_t n_last = 0;
+  if (m_req == 0) {
+    if (!large_plan(np, dtype, 2, bottom_n, &lv, &n_last)) return -1;
+    m_req = auto_m(n_last, dtype, algo);
+  }
+  if (!large_plan(np, dtype, m_req, bottom_n, &lv, &n_last)) return -1;
+  if (m_req > tridiag_max_switch_level(dtype, algo, n_last)) return -1;
+  return m_req;
+}
+
+size_t large_ws_bytes(const std::vector<LargeLevel>& lv, int64_t S, int dtype) {
+  const size_t T = elem_size(dtype);
+  const int64_t CH = large_chunk_n(dtype);
+  const int NH = ilog2_64(large_R(dtype));
+  size_t total = 0;
+  for (const LargeLevel& L : lv) {
+    total += 4 * align256((size_t)S * (size_t)(L.n >> L.kin) * T);
+    total += align256((size_t)S * (size_t)(L.n / CH - 1) * 4 * NH * T);
+  }
+  return total;
+}
+
+template <typename T>
+int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
+                  int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
+                  int64_t n_last, char* ws, cudaStream_t st) {
+  const int64_t CH = large_chunk_n(dtype);
+  const int NH = ilog2_64(large_R(dtype));
+  const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
+  struct Buf { T* a; T* b; T* c; T* d; T* h; };
+  std::vector<Buf> bufs;
+  char* p = ws;
+  for (const LargeLevel& L : lv) {
+    const size_t arr = align256((size_t)S * (size_t)(L.n >> L.kin) * sizeof(T));
+    Buf B;
+    B.a = reinterpret_cast<T*>(p); B.b = reinterpret_cast<T*>(p + arr);
+    B.c = reinterpret_cast<T*>(p + 2 * arr); B.d = reinterpret_cast<T*>(p + 3 * arr);
+    p += 4 * arr;
+    B.h = reinterpret_cast<T*>(p);
+    p += align256((size_t)S * (size_t)(L.n / CH - 1) * 4 * NH * sizeof(T));
+    bufs.push_back(B);
+  }
+  auto al = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) % 32) == 0; };
+  int launches = 0;
+  // forward: level j's inputs are the user's arrays (j = 0) or bufs[j - 1]
+  for (size_t j = 0; j < lv.size(); ++j) {
+    const LargeLevel& L = lv[j];
+    const bool first = j == 0;
+    const T* ia = first ? a : bufs[j - 1].a;
+    const T* ib = first ? b : bufs[j - 1].b;
+    const T* ic = first ? c : bufs[j - 1].c;
+    const T* id = first ? d : bufs[j - 1].d;
+    const int64_t n_real = first ? nr : L.n;
+    const int64_t ss = first ? nr : L.n;
+    const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) &&
+                     ((uint64_t)ss * sizeof(T)) % 32 == 0;
+    const Buf& B = bufs[j];
+    cudaError_t e = large_pass<T>(0, ia, ib, ic, id, nullptr, nullptr, nullptr, nullptr, nullptr,
+                                  B.h, L.n, n_real, ss, S, L.kin, vec, c_pad, st);
+    if (e == cudaSuccess)
+      e = large_pass<T>(1, ia, ib, ic, id, B.a, B.b, B.c, B.d, nullptr, B.h, L.n, n_real, ss, S,
+                        L.kin, vec, c_pad, st);
+    if (e != cudaSuccess) return (int)e;
+    launches += (L.n / CH >= 2 ? 1 : 0) + 1;
+  }
+  // on-chip solve of the reduced system, in place (x == d)
+  const Buf& Z = bufs.back();
+  const int rc = solve_device(Z.a, Z.b, Z.c, Z.d, Z.d, n_last, S, dtype, algo, m, st, Layout{1, n_last});
+  if (rc != TRIDIAG_OK) return rc;
+  launches += g_last_launches;
+  // backward: level j writes x into the user's x (j = 0) or bufs[j - 1].d
+  for (size_t jj = lv.size(); jj-- > 0;) {
+    const LargeLevel& L = lv[jj];
+    const bool first = jj == 0;
+    const T* ia = first ? a : bufs[jj - 1].a;
+    const T* ib = first ? b : bufs[jj - 1].b;
+    const T* ic = first ? c : bufs[jj - 1].c;
+    const T* id = first ? d : bufs[jj - 1].d;
+    T* ox = first ? x : bufs[jj - 1].d;
+    const int64_t n_real = first ? nr : L.n;
+    const int64_t ss = first ? nr : L.n;
+    const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) && al(ox) &&
+                     ((uint64_t)ss * sizeof(T)) % 32 == 0;
+    const cudaError_t e = large_pass<T>(2, ia, ib, ic, id, ox, nullptr, nullptr, nullptr,
+                                        bufs[jj].d, bufs[jj].h, L.n, n_real, ss, S, L.kin, vec,
+                                        c_pad, st);
+    if (e != cudaSuccess) return (int)e;
+    launches += 1;
+  }
+  g_last_launches = launches;
+  return TRIDIAG_OK;
+}
+
 }  // namespace
 
 extern "C" {
@@ -281,6 +428,7 @@ const char* tridiag_status_string(int status) {
     case TRIDIAG_ERR_OVERLAP: return "x overlaps an input (only x == d is allowed)";
     case TRIDIAG_ERR_WORKSPACE: return "workspace missing or too small";
     case TRIDIAG_ERR_STRIDE: return "invalid strides (need >= 1, one of them 1, non-overlapping)";
+    case TRIDIAG_ERR_BOTTOM_N: return "invalid bottom_n for the large-n path";
   }
   if (status > 0) return cudaGetErrorString((cudaError_t)status);
   return "unknown status";
@@ -329,6 +477,72 @@ int tridiag_solve_batched(const void* a, const void* b, const void* c, const voi
                           tridiag_stream_t stream) {
   return tridiag_solve_batched_strided(a, b, c, d, x, n, num_systems, 1, n, dtype, algo,
                                        switch_level, stream);
+}
+
+int64_t tridiag_max_n_large(int dtype, int algo) {
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return 0;
+  if (algo == TRIDIAG_CR || is_hybrid(algo)) return int64_t(1) << 30;
+  return tridiag_max_n(dtype, algo);
+}
+
+int64_t tridiag_large_chunk(int dtype) {
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return 0;
+  return large_chunk_n(dtype);
+}
+
+int64_t tridiag_large_workspace_bytes(int64_t n, int64_t num_systems, int dtype, int algo,
+                                      int switch_level, int64_t bottom_n) {
+  if (n < 1 || num_systems < 0 || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return -1;
+  if (algo < TRIDIAG_CR || algo > TRIDIAG_RD_STONE) return -1;
+  const int64_t np = pad_n(n);
+  if (np > tridiag_max_n_large(dtype, algo)) return -1;
+  const int64_t bn = resolve_bottom_n(dtype, bottom_n);
+  if (bn < 0) return -1;
+  if (np <= bn || !(algo == TRIDIAG_CR || is_hybrid(algo))) return 0;
+  const int64_t m = large_m(np, dtype, algo, switch_level, bn);
+  if (m < 0) return -1;
+  std::vector<LargeLevel> lv;
+  int64_t n_last = 0;
+  if (!large_plan(np, dtype, m, bn, &lv, &n_last)) return -1;
+  return (int64_t)large_ws_bytes(lv, num_systems, dtype);
+}
+
+int tridiag_solve_batched_large(const void* a, const void* b, const void* c, const void* d,
+                                void* x, int64_t n, int64_t num_systems, int dtype, int algo,
+                                int switch_level, int64_t bottom_n, void* workspace,
+                                int64_t workspace_bytes, tridiag_stream_t stream) {
+  g_last_launches = 0;
+  int64_t m = 0;
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, 1, n, true);
+  if (v != TRIDIAG_OK) return v;
+  const int64_t bn = resolve_bottom_n(dtype, bottom_n);
+  if (bn < 0) return TRIDIAG_ERR_BOTTOM_N;
+  const int64_t np = pad_n(n);
+  cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+  if (np <= bn) {  // fits on chip: the plain entry point's path
+    if (is_hybrid(algo) && switch_level == 0) m = auto_m(np, dtype, algo);
+    if (is_hybrid(algo) && m > tridiag_max_switch_level(dtype, algo, np)) return TRIDIAG_ERR_SWITCH_LEVEL;
+    return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, m, st, Layout{1, n});
+  }
+  if (!(algo == TRIDIAG_CR || is_hybrid(algo))) return TRIDIAG_ERR_N_TOO_LARGE;
+  m = large_m(np, dtype, algo, switch_level, bn);
+  if (m < 0) return TRIDIAG_ERR_SWITCH_LEVEL;
+  std::vector<LargeLevel> lv;
+  int64_t n_last = 0;
+  if (!large_plan(np, dtype, m, bn, &lv, &n_last)) return TRIDIAG_ERR_SWITCH_LEVEL;
+  if (num_systems == 0) return TRIDIAG_OK;
+  const size_t need = large_ws_bytes(lv, num_systems, dtype);
+  if (!workspace || workspace_bytes < 0 || (size_t)workspace_bytes < need) return TRIDIAG_ERR_WORKSPACE;
+  char* ws = static_cast<char*>(workspace);
+  if (dtype == TRIDIAG_F32)
+    return solve_large_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
+                                static_cast<const float*>(c), static_cast<const float*>(d),
+                                static_cast<float*>(x), n, num_systems, dtype, algo, m, lv, n_last,
+                                ws, st);
+  return solve_large_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
+                               static_cast<const double*>(c), static_cast<const double*>(d),
+                               static_cast<double*>(x), n, num_systems, dtype, algo, m, lv, n_last,
+                               ws, st);
 }
 
 // Host pipeline depth: three chunk buffers on three streams, so the

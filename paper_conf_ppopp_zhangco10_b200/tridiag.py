@@ -70,6 +70,14 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_last_launch_count.restype = I
         L.tridiag_phase_stamps.argtypes = [P, I64]
         L.tridiag_phase_stamps.restype = I64
+        L.tridiag_solve_batched_large.argtypes = [P, P, P, P, P, I64, I64, I, I, I, I64, P, I64, P]
+        L.tridiag_solve_batched_large.restype = I
+        L.tridiag_large_workspace_bytes.argtypes = [I64, I64, I, I, I, I64]
+        L.tridiag_large_workspace_bytes.restype = I64
+        L.tridiag_max_n_large.argtypes = [I, I]
+        L.tridiag_max_n_large.restype = I64
+        L.tridiag_large_chunk.argtypes = [I]
+        L.tridiag_large_chunk.restype = I64
         _lib = L
         return L
 
@@ -100,6 +108,31 @@ def check(status: int) -> None:
 
 def max_n(dtype, algo) -> int:
     return int(load().tridiag_max_n(_dtype_code(dtype), _algo_code(algo)))
+
+
+def max_n_large(dtype, algo) -> int:
+    return int(load().tridiag_max_n_large(_dtype_code(dtype), _algo_code(algo)))
+
+
+def large_chunk(dtype) -> int:
+    return int(load().tridiag_large_chunk(_dtype_code(dtype)))
+
+
+def large_workspace_bytes(n: int, num_systems: int, dtype, algo, switch_level=0,
+                          bottom_n=0) -> int:
+    v = int(load().tridiag_large_workspace_bytes(int(n), int(num_systems), _dtype_code(dtype),
+                                                 _algo_code(algo), int(switch_level),
+                                                 int(bottom_n)))
+    if v < 0:
+        raise ValueError("tridiag: invalid arguments for the large-n path")
+    return v
+
+
+def _pad_n(n: int) -> int:
+    p = 2
+    while p < n:
+        p <<= 1
+    return p
 
 
 def max_switch_level(dtype, algo, n: int) -> int:
@@ -185,6 +218,10 @@ def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None
     ss, es = d.stride()
     if stream is None:
         stream = torch.cuda.current_stream(d.device)
+    if (_pad_n(n) > max_n(d.dtype, algo) and es == 1 and (ss == n or S <= 1)
+            and _pad_n(n) <= max_n_large(d.dtype, algo)):
+        return solve_batched_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
+                                   stream=stream)
     with torch.cuda.device(d.device):
         if es == 1 and (ss == n or S <= 1):
             st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
@@ -194,6 +231,34 @@ def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None
             st = solve_batched_strided_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
                                            x.data_ptr(), n, S, es, max(ss, 1), d.dtype, algo,
                                            switch_level, stream.cuda_stream)
+    check(st)
+    return x
+
+
+def solve_batched_large(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, bottom_n=0,
+                        workspace=None, stream=None):
+    """tridiag_solve_batched_large: CR / CR+PCR / CR+RD for n beyond one CTA
+    (up to 2^30), contiguous (S, n) CUDA tensors.  Reduction passes of
+    log2 R CR levels shrink each system until it has <= bottom_n equations
+    (0 = tridiag_max_n), the on-chip kernels solve it, expansion passes
+    back-substitute.  ``workspace``: CUDA uint8 tensor of at least
+    large_workspace_bytes(...) bytes, allocated from torch's caching allocator
+    if None (it is used on ``stream``)."""
+    if x is None:
+        x = torch.empty_like(d)
+    _check_tensors([a, b, c, d, x], "cuda")
+    S, n = d.shape
+    if stream is None:
+        stream = torch.cuda.current_stream(d.device)
+    need = large_workspace_bytes(n, S, d.dtype, algo, switch_level, bottom_n)
+    if workspace is None:
+        with torch.cuda.device(d.device), torch.cuda.stream(stream):
+            workspace = torch.empty(max(need, 1), dtype=torch.uint8, device=d.device)
+    with torch.cuda.device(d.device):
+        st = load().tridiag_solve_batched_large(
+            a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(), x.data_ptr(), n, S,
+            _dtype_code(d.dtype), _algo_code(algo), int(switch_level), int(bottom_n),
+            workspace.data_ptr(), workspace.numel(), stream.cuda_stream)
     check(st)
     return x
 

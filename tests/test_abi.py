@@ -149,3 +149,49 @@ def test_stride_validation():
     assert strided(es=1, ss=600, S=0) == 0         # pitched rows
     assert strided(es=8, ss=1, S=0, n=8) == 0      # interleaved
     assert td.status_string(-10).startswith("invalid strides")
+
+
+def large(n, S=4, dtype=F32, algo=CR, m=0, bottom_n=0, ws=0x60000000, ws_bytes=1 << 40):
+    return int(td.load().tridiag_solve_batched_large(A, B, C, D, X, n, S, dtype, algo, m, bottom_n,
+                                                     ws, ws_bytes, None))
+
+
+def test_large_n_capacity_and_workspace():
+    """NEXT f2 (n > tridiag_max_n): CR-family up to 2^30; the
+    workspace holds 4 arrays of n/R per reduction level plus the chunk-boundary
+    heads (validation only, S = 0 or a bad argument: no launch)."""
+    for dtype in (F32, F64):
+        for algo in (CR, CR_PCR, CR_RD):
+            assert td.max_n_large(dtype, algo) == 1 << 30
+        for algo in (PCR, RD):
+            assert td.max_n_large(dtype, algo) == td.max_n(dtype, algo)
+    assert td.large_chunk(F32) == 4096 and td.large_chunk(F64) == 2048
+    # fits on chip: no workspace
+    assert td.large_workspace_bytes(8192, 10, F32, CR) == 0
+    # n = 2^20 fp32: levels 2^20 -> 2^16 -> 2^12; arrays + heads, 256-B aligned
+    S = 3
+    exp = 0
+    for nl in (1 << 20, 1 << 16):
+        exp += 4 * (-(-S * (nl >> 4) * 4 // 256) * 256)
+        exp += -(-S * (nl // 4096 - 1) * 16 * 4 // 256) * 256
+    assert td.large_workspace_bytes(1 << 20, S, F32, CR) == exp
+    # hybrids stop reducing at m: CR+PCR m = 4096 at n = 16384 is one 2-level pass
+    assert td.large_workspace_bytes(16384, 1, F32, CR_PCR, 4096) == 4 * 4096 * 4 + 256
+    with pytest.raises(ValueError):
+        td.large_workspace_bytes(1 << 31, 1, F32, CR)
+
+
+def test_large_n_validation():
+    assert large(1 << 20, S=0) == 0
+    assert large(1 << 31, S=0) == -3                       # beyond tridiag_max_n_large
+    assert large(16384, S=0, algo=PCR) == -3               # PCR / RD have no CR levels
+    assert large(16384, S=0, algo=RD) == -3
+    assert large(16384, S=0, bottom_n=1000) == -11         # not a power of two
+    assert large(16384, S=0, bottom_n=1024) == -11         # below chunk / 2
+    assert large(16384, S=0, bottom_n=16384) == -11        # above tridiag_max_n
+    assert large(16384, S=0, bottom_n=2048) == 0
+    assert large(16384, S=4, ws_bytes=16) == -9            # workspace too small
+    assert large(16384, S=4, ws=0) == -9
+    assert large(16384, S=0, algo=CR_PCR, m=8192) == -7    # m > max inner m
+    assert large(16384, S=0, algo=CR_PCR, m=3) == -7
+    assert td.status_string(-11).startswith("invalid bottom_n")

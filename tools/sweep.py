@@ -8,6 +8,9 @@
          launches over rotating buffer sets -> us per batch).
   c3     ADI-style 4096 x 4096, fp32 and fp64, all algorithms that fit.
   c4     2^20 x 256 fp32 on one GPU (the W = 1 point of the scaling row).
+  large  n = 2^14 .. 2^24 beyond one CTA (NEXT f2), S*n = 2^26 (fp32) / 2^25
+         (fp64), CR / CR+PCR / CR+RD through the reduction passes: algorithmic
+         GB/s (5nT) and the pass model's traffic (each level read twice).
 
 Writes one JSON object per point to stdout.  Timing: CUDA events on the
 launching stream, warm-up first, working set >= 4x L2 via rotating buffer sets.
@@ -199,6 +202,47 @@ def c4(args):
               "frac_of_peak": per / med / 1e9 / PEAK})
 
 
+def large_traffic(n, T, LR, bottom):
+    """HBM bytes per system of the large-n pipeline (tridiag_large.cuh):
+    per level, reduce reads 4n writes 4n/R, expand reads 4n + n/R writes n
+    (heads: 4 R T per chunk boundary); the bottom solve 5 n_last T."""
+    tot = 0
+    cur = n
+    while cur > bottom:
+        chunks = cur // (256 * (1 << LR))
+        nxt = cur >> LR
+        tot += (4 * cur + 4 * nxt) + (4 * cur + nxt + cur) + 4 * (1 << LR) * max(chunks - 1, 0)
+        cur = nxt
+    return (tot + 5 * cur) * T
+
+
+def large(args):
+    for dts in ("f32", "f64"):
+        dt = torch.float32 if dts == "f32" else torch.float64
+        T = 4 if dts == "f32" else 8
+        LR = 4 if dts == "f32" else 3
+        total = (1 << 26) if dts == "f32" else (1 << 25)
+        for ln in range(14, 25):
+            n = 1 << ln
+            S = max(1, total // n)
+            for algo in ("cr", "cr_pcr", "cr_rd"):
+                fam = "rdw" if algo == "cr_rd" else "dd"
+                sets, per = make_sets(fam, S, n, dt, 4 * L2_BYTES)
+                med, mn = time_point(sets, algo, 0, steps=args.steps)
+                model = large_traffic(n, T, LR, td.max_n(dt, "cr")) * S
+                row = {"config": "large", "dtype": dts, "n": n, "S": S, "algo": algo,
+                       "time_family": fam, "ms_median": med * 1e3, "ms_min": mn * 1e3,
+                       "systems_per_s": S / med, "gbs": per / med / 1e9,
+                       "frac_of_peak": per / med / 1e9 / PEAK,
+                       "model_bytes_per_5nT": model / per,
+                       "model_gbs": model / med / 1e9, "model_frac": model / med / 1e9 / PEAK}
+                if not args.no_acc:
+                    row["acc"] = accuracy(fam, n, dt, algo, 0, S=2)
+                emit(row)
+                del sets
+                torch.cuda.empty_cache()
+
+
 def adi(args):
     """ADI-style 2D sweeps on NY x NX row-major grids: the row sweep solves NY
     contiguous systems of n = NX, the column sweep NX interleaved systems of
@@ -229,7 +273,7 @@ def adi(args):
 
 if __name__ == "__main__":
     p = argparse.ArgumentParser()
-    p.add_argument("configs", nargs="+", choices=["c2", "c3", "c4", "c5", "adi"])
+    p.add_argument("configs", nargs="+", choices=["c2", "c3", "c4", "c5", "adi", "large"])
     p.add_argument("--steps", type=int, default=30)
     p.add_argument("--no-acc", action="store_true")
     a = p.parse_args()
