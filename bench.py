@@ -355,7 +355,7 @@ def main():
         # --- e2e: host (pinned) buffers through the C ABI, copies inside the timed region
         ha, hb, hc, hd = [t.cpu().pin_memory() for t in (a, b, c, d)]
         hx = torch.empty_like(hd).pin_memory()
-        chunk = 8192
+        chunk = 16384
         ws = torch.empty(td.host_workspace_bytes(n, dt, chunk), dtype=torch.uint8, device="cuda")
         td.solve_batched_host(ha, hb, hc, hd, hx, algo=args.algo, switch_level=m,
                               chunk_systems=chunk, workspace=ws)
@@ -400,34 +400,41 @@ def main():
         del a, b, c, d, x
         torch.cuda.empty_cache()
         other = {}
-        for name, dts, nn, SS, layout in (("c3_f32_4096x4096_rows", "f32", 4096, 4096, "rows"),
-                                          ("c3_f32_4096x4096_columns", "f32", 4096, 4096, "cols"),
-                                          ("c3_f64_4096x4096_rows", "f64", 4096, 4096, "rows"),
-                                          ("c4_f32_1048576x256", "f32", 256, 1 << 20, "rows"),
-                                          ("c5_f32_16384x8192", "f32", 8192, 16384, "rows")):
+        # plus RD at C3 (CTA-blocked scan; RD-stable rdw input) and the large-n
+        # passes (NEXT f2) at S * n = 2^26.
+        for name, dts, nn, SS, layout, oalgo, fam in (
+                ("c3_f32_4096x4096_rows", "f32", 4096, 4096, "rows", "cr_pcr", "dd"),
+                ("c3_f32_4096x4096_columns", "f32", 4096, 4096, "cols", "cr_pcr", "dd"),
+                ("c3_f64_4096x4096_rows", "f64", 4096, 4096, "rows", "cr_pcr", "dd"),
+                ("c3_f32_4096x4096_rows_rd", "f32", 4096, 4096, "rows", "rd", "rdw"),
+                ("c4_f32_1048576x256", "f32", 256, 1 << 20, "rows", "cr_pcr", "dd"),
+                ("c5_f32_16384x8192", "f32", 8192, 16384, "rows", "cr_pcr", "dd"),
+                ("large_f32_64x1048576", "f32", 1 << 20, 64, "rows", "cr_pcr", "dd"),
+                ("large_f64_32x1048576", "f64", 1 << 20, 32, "rows", "cr_pcr", "dd")):
             dtt = torch.float32 if dts == "f32" else torch.float64
             TT = 4 if dts == "f32" else 8
             sets = []
             nsets = max(1, -(-4 * 126 * 2**20 // (5 * nn * SS * TT)))
             for kk in range(nsets):
-                g = inputs.generate("dd", SS, nn, dtt, s0=kk * SS, device="cuda")
+                g = inputs.generate(fam, SS, nn, dtt, s0=kk * SS, device="cuda")
                 if layout == "cols":
                     g = [t.t().contiguous().t() for t in g]
                 sets.append((*g, torch.empty_like(g[3])))
             steps = max(5, args.steps // 10)
             for i in range(3):
-                td.solve_batched(*sets[i % nsets], algo="cr_pcr", stream=stream)
+                td.solve_batched(*sets[i % nsets], algo=oalgo, stream=stream)
             torch.cuda.synchronize()
             e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
             e0.record(stream)
             for i in range(steps):
-                td.solve_batched(*sets[i % nsets], algo="cr_pcr", stream=stream)
+                td.solve_batched(*sets[i % nsets], algo=oalgo, stream=stream)
             e1.record(stream)
             torch.cuda.synchronize()
             tt = reduce_max(e0.elapsed_time(e1) / 1e3 / steps)
             gbs = 5 * nn * TT * SS / tt / 1e9
             other[name] = {"systems_per_s_per_gpu": SS / tt, "gbs_per_gpu": gbs,
-                           "frac_of_peak": gbs / peak, "layout": layout, "algo": "cr_pcr"}
+                           "frac_of_peak": gbs / peak, "layout": layout, "algo": oalgo,
+                           "family": fam}
             del sets
             torch.cuda.empty_cache()
         line["other_configs"] = other

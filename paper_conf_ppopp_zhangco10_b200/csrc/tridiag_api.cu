@@ -53,12 +53,13 @@ bool cta_plan(int dtype, int64_t n);
 int auto_m(int64_t n, int dtype, int algo) {
   if (!is_hybrid(algo)) return 0;
   const int64_t P = lanes_per_system(dtype, n);
-  // CTA plans (n > 32 R): CR+PCR keeps m = 32 (one warp-level PCR); CR+RD
-  // takes m = n / R, one survivor per lane for the CTA-wide register-blocked
-  // scan, 0.90-0.996 of HBM vs 0.74-0.91 at m = 32 (profiles/r01_rd_tune2.txt).
-  int64_t m = algo == TRIDIAG_CR_PCR ? std::min<int64_t>(P, 32)
-            : cta_plan(dtype, n)     ? n / plan_for(dtype, n).R
-                                     : std::min<int64_t>(P, 8);
+  // CTA plans (n > 32 R): m = 32 for both hybrids.  For CR+RD, m = n / R (one
+  // survivor per lane for the CTA-wide blocked scan) is 8-25% faster
+  // (profiles/r01_rd_tune2.txt) but RD's error grows with m (R24: POI fp32
+  // 2e-5 at m = 32, ~1e-3 at m = 256), so the table keeps the accurate m and
+  // the fast one is the caller's choice.
+  int64_t m = (algo == TRIDIAG_CR_PCR || cta_plan(dtype, n)) ? std::min<int64_t>(P, 32)
+                                                             : std::min<int64_t>(P, 8);
   if (m < 2) m = 2;
   if (m > n) m = n;
   return (int)m;

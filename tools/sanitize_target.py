@@ -22,6 +22,11 @@ CASES = [
     (torch.float32, 100, 33, "cr_pcr", 0, "contig"),     # ragged n (general path)
     (torch.float32, 256, 30, "cr_pcr", 0, "column"),     # interleaved tile kernel
     (torch.float32, 1024, 12, "cr", 0, "column"),        # CTA general strided path
+    (torch.float32, 2048, 6, "rd", 0, "contig"),         # TMA CTA kernel, CTA-blocked RD scan
+    (torch.float64, 1024, 5, "cr_rd", 256, "contig"),    # same, k = 2 in-lane levels
+    (torch.float32, 1000, 7, "rd", 0, "contig"),         # CTA-blocked RD, staged ragged path
+    (torch.float32, 16384, 2, "cr_pcr", 0, "contig"),    # large-n passes
+    (torch.float64, 12289, 2, "cr_rd", 0, "contig"),     # large-n passes, ragged, RD inner
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
@@ -29,7 +34,7 @@ bad = 0
 for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
     if only is not None and idx != only:
         continue
-    fam = "poi" if algo in ("rd", "cr_rd") else "dd"
+    fam = "rdw" if algo in ("rd", "cr_rd") else "dd"
     a, b, c, d = inputs.generate(fam, S, n, dt, device="cuda")
     if layout == "column":
         views = [t.t().contiguous().t() for t in (a, b, c, d)]
