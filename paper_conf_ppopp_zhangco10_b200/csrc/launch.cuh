@@ -14,25 +14,26 @@ template <typename T, int R, int INNER, int KB>
 cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
                             int64_t S, int k, cudaStream_t st, int64_t n_real, Layout L) {
   const int P = (int)(n / R);
-  const int G = std::max(8, 32 / P);
-  const int threads = G * P;
-  // 16-byte vector row segments when every row segment is 16-byte aligned
-  auto a16 = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) & 15) == 0; };
-  // (each thread moves R / V row segments: needs R >= V = 16 / sizeof(T))
-  const int vec16 = R * sizeof(T) >= 16 && a16(a) && a16(b) && a16(c) && a16(d) && a16(x) &&
-                    ((uint64_t)L.es * sizeof(T)) % 16 == 0 ? 1 : 0;
-  const size_t smem = (size_t)4 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
+  const int lp = ilog2c(P);
+  const int threads = 1 << tdg::ilv_log_threads(lp);
+  const int G = threads / P;  // a tile is threads * R elements per array
+  const size_t smem = (size_t)5 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
   if (smem > 227 * 1024) return cudaErrorInvalidValue;
   int dev = 0;
   cudaGetDevice(&dev);
-  auto kern = tdg::tdg_ileave_kernel<T, R, INNER, KB>;
+  // compile-time geometry for the lane counts the plans use (P = 4 .. 32)
+  auto kern = lp == 5 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 5>
+            : lp == 4 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 4>
+            : lp == 3 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 3>
+            : lp == 2 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 2>
+                      : tdg::tdg_ileave_kernel<T, R, INNER, KB, -1>;
   const int occ = occupancy(dev, kern, threads, smem);
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t tiles = (S + G - 1) / G;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)device_sms(dev) * occ));
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
-  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, ilog2c(P),
-                                              ilog2c(G), (int)n_real, c_pad, (long long)L.es, vec16);
+  kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, lp,
+                                              (int)n_real, c_pad, (long long)L.es);
   g_last_launches = 1;
   return cudaGetLastError();
 }

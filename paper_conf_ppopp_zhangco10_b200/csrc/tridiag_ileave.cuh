@@ -27,110 +27,153 @@ __host__ __device__ constexpr int ilv_tile_elems(int n_pad, int G) {
   return n_pad * G + (n_pad >> 4) + G;
 }
 
-template <typename T, int R, int INNER, int KB>
-__global__ void __launch_bounds__(256)
+// ---- asynchronous 4 / 8-byte global -> shared copies (LDGSTS) ----
+template <typename T>
+__device__ __forceinline__ void cp_async_elem(T* dst, const T* src) {
+  const unsigned s = (unsigned)__cvta_generic_to_shared(dst);
+  if constexpr (sizeof(T) == 4)
+    asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(s), "l"(src) : "memory");
+  else
+    asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(s), "l"(src) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+__device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wait_group 0;" ::: "memory"); }
+
+// Tile geometry.  NT = 2^ilv_log_threads threads; P = 2^LP lanes per
+// system, G = NT / P systems per tile, ROWS = P R rows.  LP >= 0 makes every shared-memory
+// offset a compile-time immediate (the kernel is integer-bound otherwise);
+// LP = -1 takes log2P at run time.
+// 512 threads (G = 16 systems, 64-byte fp32 row segments) at P = 32, where
+// 32-byte segments over-fetch from DRAM; 256 threads for smaller P.
+__host__ __device__ constexpr int ilv_log_threads(int lp) { return lp == 5 ? 9 : 8; }
+template <int LP>
+struct IlvGeom {
+  int lp, lnt;
+  __device__ __forceinline__ explicit IlvGeom(int log2P)
+      : lp(LP >= 0 ? LP : log2P), lnt(ilv_log_threads(LP >= 0 ? LP : log2P)) {}
+  __device__ __forceinline__ int P() const { return 1 << lp; }
+  __device__ __forceinline__ int lg() const { return lnt - lp; }
+  __device__ __forceinline__ int G() const { return 1 << (lnt - lp); }
+};
+
+// Issue the copies of one tile: rows [row0, row0 + ROWS) of systems
+// [t0, t0 + G) into the padded tile.  Thread tid owns system g = tid % G and
+// rows r0 + P j (r0 = tid / G < P, j < R), so consecutive threads read
+// consecutive systems of a row (whole 32-byte sectors); every offset advances
+// by a constant.  Padding (rows >= n_real, systems >= S, reading R26) and
+// c_{n_real-1} <- c_pad are plain shared stores.
+template <typename T, int R, int LP, bool COPY_D>
+__device__ __forceinline__ void ilv_issue(const T* a, const T* b, const T* c, const T* d, T* tile,
+                                          int TE, long long t0, long long S, int row0, int n_real,
+                                          long long es, const IlvGeom<LP>& Gm, T c_pad) {
+  const int G = Gm.G(), P = Gm.P();
+  const int g = threadIdx.x & (G - 1);
+  const int r0 = threadIdx.x >> Gm.lg();
+  const bool sys_ok = t0 + g < S;
+  const long long off0 = t0 + g + (long long)(row0 + r0) * es;
+  const T* pa = a + off0;
+  const T* pb = b + off0;
+  const T* pc = c + off0;
+  const T* pd = d + off0;
+  const long long step = (long long)P * es;
+  unsigned so = (unsigned)__cvta_generic_to_shared(tile) + (unsigned)(r0 * G + g) * sizeof(T);
+  const unsigned TB = (unsigned)TE * sizeof(T);
+  const bool all_rows = row0 + P * R <= n_real - 1;  // no padding row, no c_{n_real-1} here
+#pragma unroll 4
+  for (int j = 0; j < R; ++j, pa += step, pb += step, pc += step, pd += step) {
+    // (r0 + P j) >> 4 == (P j) >> 4 + (r0 >> 4) for P | 16 or 16 | P
+    const int r = r0 + P * j;
+    const unsigned sj = so + (unsigned)(P * j * G + (r >> 4)) * sizeof(T);
+    const int row = row0 + r;
+    if (sys_ok && (all_rows || row < n_real)) {
+      if constexpr (sizeof(T) == 4) {
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj), "l"(pa) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + TB), "l"(pb) : "memory");
+        if (all_rows || row != n_real - 1)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + 2 * TB), "l"(pc) : "memory");
+        if (COPY_D)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + 3 * TB), "l"(pd) : "memory");
+      } else {
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj), "l"(pa) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + TB), "l"(pb) : "memory");
+        if (all_rows || row != n_real - 1)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + 2 * TB), "l"(pc) : "memory");
+        if (COPY_D)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + 3 * TB), "l"(pd) : "memory");
+      }
+      if (!all_rows && row == n_real - 1) tile[2 * TE + ilv_off(r, g, G)] = c_pad;
+    } else {
+      const int o = ilv_off(r, g, G);
+      tile[o] = T(0); tile[TE + o] = T(1); tile[2 * TE + o] = c_pad;
+      if (COPY_D) tile[3 * TE + o] = T(0);
+    }
+  }
+  cp_async_commit();
+}
+
+// Write the tile's x back: same element mapping, coalesced.
+template <typename T, int R, int LP>
+__device__ __forceinline__ void ilv_writeback(T* x, const T* tX, long long t0, long long S, int row0,
+                                              int n_real, long long es, const IlvGeom<LP>& Gm) {
+  const int G = Gm.G(), P = Gm.P();
+  const int g = threadIdx.x & (G - 1);
+  const int r0 = threadIdx.x >> Gm.lg();
+  if (t0 + g >= S) return;
+  T* dst = x + t0 + g + (long long)(row0 + r0) * es;
+  const long long step = (long long)P * es;
+  const T* srcp = tX + r0 * G + g;
+  const bool all_rows = row0 + P * R <= n_real;
+#pragma unroll 4
+  for (int j = 0; j < R; ++j, dst += step) {
+    const int r = r0 + P * j;
+    if (all_rows || row0 + r < n_real) *dst = srcp[P * j * G + (r >> 4)];
+  }
+}
+
+// Interleaved solve, n <= 32 R: NT threads, P = n / R lanes per system,
+// G = NT / P systems per tile (NT = 512 at P = 32: 64-byte fp32 / 128-byte
+// fp64 row segments; else 256).  One input tile plus an x tile: as soon as the
+// lanes hold tile i in registers the copies of tile i+1 are issued into the
+// same buffer (no registers held while they fly) and overlap the solve; x
+// leaves through the x tile.  5 NT R elements of shared memory: 1 CTA of 16
+// warps (NT = 512) or 2 CTAs of 8 warps per SM.
+template <typename T, int R, int INNER, int KB, int LP>
+__global__ void __launch_bounds__(LP == 5 ? 512 : 256, LP == 5 ? 1 : 2)
 tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                  const T* d, T* x, int n, long long S, int k, int log2P, int log2G, int n_real,
-                  T c_pad, long long es, int vec16) {
+                  const T* d, T* x, int n, long long S, int k, int log2P, int n_real, T c_pad,
+                  long long es) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   T* tile = reinterpret_cast<T*>(smem_raw);
-  const int G = 1 << log2G;
-  const int TE = ilv_tile_elems(n, G);
-  T* tA = tile;
-  T* tB = tile + TE;
-  T* tC = tile + 2 * TE;
-  T* tD = tile + 3 * TE;
-  const int P = 1 << log2P;
-  const int NT = blockDim.x;  // = G * P
-  const int g = threadIdx.x >> log2P;
+  const IlvGeom<LP> Gm(log2P);
+  const int G = Gm.G(), P = Gm.P();
+  const int TE = ilv_tile_elems(P * R, G);
+  T* tX = tile + 4 * TE;
+  const int g = threadIdx.x >> Gm.lp;
   const int ls = threadIdx.x & (P - 1);
-  // Row-segment mapping for the coalesced phases: V consecutive systems per
-  // thread (one 16-byte vector when aligned, else V = 1).
-  constexpr int V16 = 16 / (int)sizeof(T);
-  const int V = vec16 ? V16 : 1;
-  const int lv = vec16 ? (V16 == 4 ? 2 : 1) : 0;
-  const int qpr = G >> lv;                     // threads per row segment
-  const int lq = log2G - lv;
-  const int q = threadIdx.x & (qpr - 1);       // which V-group of the row
-  const int r0 = threadIdx.x >> lq;            // first row of this thread
-  const int RS = NT >> lq;                     // rows per sweep
-  const long long step = (long long)RS * es;
-  for (long long t0 = (long long)blockIdx.x * G; t0 < S; t0 += (long long)gridDim.x * G) {
-    const long long s0 = t0 + q * V;           // first system of this thread's group
-    // ---- coalesced load of the tile ----
-    {
-      long long e = s0 + (long long)r0 * es;
-      for (int r = r0; r < n; r += RS, e += step) {
-        const int o = ilv_off(r, q * V, G);
-        if (r < n_real && s0 + V <= S) {
-          T va[V16], vb[V16], vc[V16], vd[V16];
-          if (vec16) {
-            if constexpr (sizeof(T) == 4) {
-              const float4 A4 = __ldg(reinterpret_cast<const float4*>(a + e));
-              const float4 B4 = __ldg(reinterpret_cast<const float4*>(b + e));
-              const float4 C4 = __ldg(reinterpret_cast<const float4*>(c + e));
-              const float4 D4 = *reinterpret_cast<const float4*>(d + e);
-              va[0] = A4.x; va[1] = A4.y; va[2] = A4.z; va[3] = A4.w;
-              vb[0] = B4.x; vb[1] = B4.y; vb[2] = B4.z; vb[3] = B4.w;
-              vc[0] = C4.x; vc[1] = C4.y; vc[2] = C4.z; vc[3] = C4.w;
-              vd[0] = D4.x; vd[1] = D4.y; vd[2] = D4.z; vd[3] = D4.w;
-            } else {
-              const double2 A2 = __ldg(reinterpret_cast<const double2*>(a + e));
-              const double2 B2 = __ldg(reinterpret_cast<const double2*>(b + e));
-              const double2 C2 = __ldg(reinterpret_cast<const double2*>(c + e));
-              const double2 D2 = *reinterpret_cast<const double2*>(d + e);
-              va[0] = A2.x; va[1] = A2.y; vb[0] = B2.x; vb[1] = B2.y;
-              vc[0] = C2.x; vc[1] = C2.y; vd[0] = D2.x; vd[1] = D2.y;
-            }
-#pragma unroll
-            for (int j = 0; j < V16; ++j) {
-              tA[o + j] = va[j]; tB[o + j] = vb[j];
-              tC[o + j] = (r == n_real - 1) ? c_pad : vc[j];
-              tD[o + j] = vd[j];
-            }
-          } else {
-            tA[o] = a[e]; tB[o] = b[e]; tC[o] = (r == n_real - 1) ? c_pad : c[e]; tD[o] = d[e];
-          }
-        } else {
-          for (int j = 0; j < V; ++j) {
-            const bool ok = r < n_real && s0 + j < S;
-            tA[o + j] = ok ? a[e + j] : T(0);
-            tB[o + j] = ok ? b[e + j] : T(1);
-            tC[o + j] = ok ? ((r == n_real - 1) ? c_pad : c[e + j]) : c_pad;
-            tD[o + j] = ok ? d[e + j] : T(0);
-          }
-        }
-      }
-    }
-    __syncthreads();
+  // lane-blocked rows ls R + q of system g: offset base + q G (R | 16 or 16 | R)
+  const int base = ls * R * G + g + ((ls * R) >> 4);
+  const long long tiles = (S + G - 1) / G;
+  long long t = blockIdx.x;
+  if (t < tiles) ilv_issue<T, R, LP, true>(a, b, c, d, tile, TE, t * G, S, 0, n_real, es, Gm, c_pad);
+  for (; t < tiles; t += gridDim.x) {
+    cp_async_wait_all();
+    __syncthreads();  // tile t landed; the x tile's previous write-back is done
     T ra[R], rb[R], rc[R], rd[R];
 #pragma unroll
-    for (int t = 0; t < R; ++t) {
-      const int o = ilv_off(ls * R + t, g, G);
-      ra[t] = tA[o]; rb[t] = tB[o]; rc[t] = tC[o]; rd[t] = tD[o];
+    for (int q = 0; q < R; ++q) {
+      const int o = base + q * G;
+      ra[q] = tile[o]; rb[q] = tile[TE + o]; rc[q] = tile[2 * TE + o]; rd[q] = tile[3 * TE + o];
     }
+    __syncthreads();  // every lane holds its rows: the tile buffer is free
+    const long long tn = t + gridDim.x;
+    if (tn < tiles) ilv_issue<T, R, LP, true>(a, b, c, d, tile, TE, tn * G, S, 0, n_real, es, Gm, c_pad);
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
 #pragma unroll
-    for (int t = 0; t < R; ++t) tD[ilv_off(ls * R + t, g, G)] = rd[t];
+    for (int q = 0; q < R; ++q) tX[base + q * G] = rd[q];
     __syncthreads();
-    {
-      long long e = s0 + (long long)r0 * es;
-      for (int r = r0; r < n_real; r += RS, e += step) {
-        const int o = ilv_off(r, q * V, G);
-        if (vec16 && s0 + V <= S) {
-          if constexpr (sizeof(T) == 4)
-            *reinterpret_cast<float4*>(x + e) = make_float4(tD[o], tD[o + 1], tD[o + 2], tD[o + 3]);
-          else
-            *reinterpret_cast<double2*>(x + e) = make_double2(tD[o], tD[o + 1]);
-        } else {
-          for (int j = 0; j < V; ++j)
-            if (s0 + j < S) x[e + j] = tD[o + j];
-        }
-      }
-    }
-    __syncthreads();
+    ilv_writeback<T, R, LP>(x, tX, t * G, S, 0, n_real, es, Gm);
   }
 }
 
