@@ -406,6 +406,7 @@ def main():
                 ("c3_f32_4096x4096_rows", "f32", 4096, 4096, "rows", "cr_pcr", "dd"),
                 ("c3_f32_4096x4096_columns", "f32", 4096, 4096, "cols", "cr_pcr", "dd"),
                 ("c3_f64_4096x4096_rows", "f64", 4096, 4096, "rows", "cr_pcr", "dd"),
+                ("c3_f64_4096x4096_columns", "f64", 4096, 4096, "cols", "cr_pcr", "dd"),
                 ("c3_f32_4096x4096_rows_rd", "f32", 4096, 4096, "rows", "rd", "rdw"),
                 ("c4_f32_1048576x256", "f32", 256, 1 << 20, "rows", "cr_pcr", "dd"),
                 ("c5_f32_16384x8192", "f32", 8192, 16384, "rows", "cr_pcr", "dd"),

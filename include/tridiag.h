@@ -201,6 +201,54 @@ int64_t tridiag_max_n_large(int dtype, int algo);
 /* Equations per reduction chunk (one CTA) of the large-n passes. */
 int64_t tridiag_large_chunk(int dtype);
 
+/*
+ * tridiag_solve_batched_strided_large -- tridiag_solve_batched_strided with a
+ * workspace, for strided layouts whose systems do not fit one CTA's on-chip
+ * kernel in that layout (SURVEY.md 8(f) NEXT f1 + f2).  Same arguments,
+ * layout rules (element (s, i) at ptr[s * sys_stride + i * elem_stride]),
+ * semantics and errors as tridiag_solve_batched_strided, plus bottom_n /
+ * workspace as in tridiag_solve_batched_large; n_pad up to
+ * tridiag_max_n_large for CR and the hybrids.
+ *
+ * Rows (elem_stride == 1, contiguous or pitched): exactly
+ * tridiag_solve_batched_large (row reduction passes while n_pad > bottom_n).
+ *
+ * Interleaved columns (sys_stride == 1, elem_stride >= num_systems: the ADI
+ * column sweep): for CR, CR+PCR and CR+RD with
+ * n_pad > bottom_n, column reduction passes of log2 R CR levels
+ * -- one CTA per 32 consecutive systems x W R rows, every warp access one
+ * coalesced row segment of 32 systems -- write the surviving equations, still
+ * interleaved (element stride num_systems), to the workspace until at most
+ * bottom_n remain; the interleaved on-chip kernel solves them; expansion
+ * passes back-substitute and write x.  bottom_n: 0 = 32 R
+ * (512 fp32 / 256 fp64, the interleaved kernel's capacity), else a power of
+ * two in [tridiag_column_chunk(dtype) / 2, 32 R].  HBM traffic about
+ * 9.6 n T per system (each level read twice) against 5 n T on chip, but every
+ * access is a full row segment where the on-chip strided kernel reads 4-byte
+ * pieces of 32-byte sectors.  Hybrid default m: the contiguous solve's tuned
+ * m of the full size, so results are bitwise identical to
+ * tridiag_solve_batched on the transposed data.  PCR, RD, RD_STONE, and
+ * hybrid m that the passes cannot reach, take the on-chip strided path
+ * (no workspace).
+ *
+ * workspace   caller-owned device buffer of at least
+ *             tridiag_strided_large_workspace_bytes(...) bytes (0 when no
+ *             passes run; NULL allowed then); 256-byte aligned.
+ * Asynchronous on `stream`; x == d allowed.
+ */
+int tridiag_solve_batched_strided_large(const void* a, const void* b, const void* c,
+                                        const void* d, void* x, int64_t n, int64_t num_systems,
+                                        int64_t elem_stride, int64_t sys_stride, int dtype,
+                                        int algo, int switch_level, int64_t bottom_n,
+                                        void* workspace, int64_t workspace_bytes,
+                                        tridiag_stream_t stream);
+/* Workspace bytes of tridiag_solve_batched_strided_large; -1 if invalid. */
+int64_t tridiag_strided_large_workspace_bytes(int64_t n, int64_t num_systems,
+                                              int64_t elem_stride, int64_t sys_stride, int dtype,
+                                              int algo, int switch_level, int64_t bottom_n);
+/* Rows per column-pass chunk (one CTA: W R rows of 32 systems). */
+int64_t tridiag_column_chunk(int dtype);
+
 /* Human-readable text of a status code (static storage, never NULL). */
 const char* tridiag_status_string(int status);
 

@@ -332,7 +332,7 @@ size_t large_ws_bytes(const std::vector<LargeLevel>& lv, int64_t S, int dtype) {
 template <typename T>
 int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
                   int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
-                  int64_t n_last, char* ws, cudaStream_t st) {
+                  int64_t n_last, char* ws, cudaStream_t st, int64_t ss0) {
   const int64_t CH = large_chunk_n(dtype);
   const int NH = ilog2_64(large_R(dtype));
   const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
@@ -360,7 +360,7 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     const T* ic = first ? c : bufs[j - 1].c;
     const T* id = first ? d : bufs[j - 1].d;
     const int64_t n_real = first ? nr : L.n;
-    const int64_t ss = first ? nr : L.n;
+    const int64_t ss = first ? ss0 : L.n;
     const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) &&
                      ((uint64_t)ss * sizeof(T)) % 32 == 0;
     const Buf& B = bufs[j];
@@ -387,7 +387,7 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     const T* id = first ? d : bufs[jj - 1].d;
     T* ox = first ? x : bufs[jj - 1].d;
     const int64_t n_real = first ? nr : L.n;
-    const int64_t ss = first ? nr : L.n;
+    const int64_t ss = first ? ss0 : L.n;
     const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) && al(ox) &&
                      ((uint64_t)ss * sizeof(T)) % 32 == 0;
     const cudaError_t e = large_pass<T>(2, ia, ib, ic, id, ox, nullptr, nullptr, nullptr,
@@ -397,6 +397,170 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     launches += 1;
   }
   g_last_launches = launches;
+  return TRIDIAG_OK;
+}
+
+// ---------------------------------------------------------------------------
+// Interleaved layouts with n > 32 R (the ADI column sweep, NEXT f1 + f2):
+// column reduction passes (tridiag_colpass.cuh) until the system has at most
+// col_bottom equations, the interleaved on-chip kernel on the reduced system
+// (still interleaved, element stride S, in the workspace), expansion passes.
+// ---------------------------------------------------------------------------
+int64_t col_chunk_n(int dtype) { return dtype == TRIDIAG_F64 ? col_chunk<double>() : col_chunk<float>(); }
+int64_t col_bottom_max(int dtype) { return 32 * large_R(dtype); }  // interleaved kernel capacity
+
+int64_t resolve_col_bottom(int dtype, int64_t bottom_n) {
+  if (bottom_n == 0) return col_bottom_max(dtype);
+  if (!is_pow2(bottom_n) || bottom_n < col_chunk_n(dtype) / 2 || bottom_n > col_bottom_max(dtype)) return -1;
+  return bottom_n;
+}
+
+bool col_plan(int64_t np, int dtype, int64_t m, int64_t bottom, std::vector<LargeLevel>* lv,
+              int64_t* n_last) {
+  const int LR = ilog2_64(large_R(dtype));
+  const int64_t CH = col_chunk_n(dtype);
+  lv->clear();
+  int64_t cur = np;
+  while (cur > bottom) {
+    const int kin = std::min(LR, ilog2_64(cur / m));
+    if (kin < 1 || cur % CH != 0) return false;
+    lv->push_back({cur, kin});
+    cur >>= kin;
+  }
+  *n_last = cur;
+  return !lv->empty();
+}
+
+// m of a column-pass solve (CR 2; hybrids the caller's m, else the tuned m of
+// the full size -- the same default as the contiguous solve -- or, beyond the
+// on-chip sizes, of the reduced size); -1 when no pass plan exists.
+int64_t col_m(int64_t np, int dtype, int algo, int64_t m_req, int64_t bottom,
+              std::vector<LargeLevel>* lv, int64_t* n_last) {
+  if (algo == TRIDIAG_CR) {
+    if (!col_plan(np, dtype, 2, bottom, lv, n_last)) return -1;
+    return 2;
+  }
+  if (!is_hybrid(algo)) return -1;
+  if (m_req == 0) {
+    if (np <= max_n_cr(dtype)) {
+      m_req = auto_m(np, dtype, algo);
+    } else {
+      if (!col_plan(np, dtype, 2, bottom, lv, n_last)) return -1;
+      m_req = auto_m(*n_last, dtype, algo);
+    }
+  }
+  if (!col_plan(np, dtype, m_req, bottom, lv, n_last)) return -1;
+  if (m_req > tridiag_max_switch_level(dtype, algo, *n_last)) return -1;
+  return m_req;
+}
+
+size_t col_ws_bytes(const std::vector<LargeLevel>& lv, int64_t S, int dtype) {
+  const size_t T = elem_size(dtype);
+  size_t total = 0;
+  for (const LargeLevel& L : lv) total += 4 * align256((size_t)S * (size_t)(L.n >> L.kin) * T);
+  return total;
+}
+
+template <typename T>
+int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
+                int64_t es, int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
+                int64_t n_last, char* ws, cudaStream_t st) {
+  const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
+  struct Buf { T* a; T* b; T* c; T* d; };
+  std::vector<Buf> bufs;
+  char* p = ws;
+  for (const LargeLevel& L : lv) {
+    const size_t arr = align256((size_t)S * (size_t)(L.n >> L.kin) * sizeof(T));
+    Buf B;
+    B.a = reinterpret_cast<T*>(p); B.b = reinterpret_cast<T*>(p + arr);
+    B.c = reinterpret_cast<T*>(p + 2 * arr); B.d = reinterpret_cast<T*>(p + 3 * arr);
+    p += 4 * arr;
+    bufs.push_back(B);
+  }
+  int launches = 0;
+  for (size_t j = 0; j < lv.size(); ++j) {
+    const LargeLevel& L = lv[j];
+    const bool first = j == 0;
+    const T* ia = first ? a : bufs[j - 1].a;
+    const T* ib = first ? b : bufs[j - 1].b;
+    const T* ic = first ? c : bufs[j - 1].c;
+    const T* id = first ? d : bufs[j - 1].d;
+    const Buf& B = bufs[j];
+    const cudaError_t e = col_pass<T>(1, ia, ib, ic, id, B.a, B.b, B.c, B.d, nullptr, L.n,
+                                      first ? nr : L.n, first ? es : S, S, S, L.kin, c_pad, st);
+    if (e != cudaSuccess) return (int)e;
+    launches += 1;
+  }
+  const Buf& Z = bufs.back();
+  const int rc = solve_device(Z.a, Z.b, Z.c, Z.d, Z.d, n_last, S, dtype, algo, m, st, Layout{S, 1});
+  if (rc != TRIDIAG_OK) return rc;
+  launches += g_last_launches;
+  for (size_t jj = lv.size(); jj-- > 0;) {
+    const LargeLevel& L = lv[jj];
+    const bool first = jj == 0;
+    const T* ia = first ? a : bufs[jj - 1].a;
+    const T* ib = first ? b : bufs[jj - 1].b;
+    const T* ic = first ? c : bufs[jj - 1].c;
+    const T* id = first ? d : bufs[jj - 1].d;
+    T* ox = first ? x : bufs[jj - 1].d;
+    const cudaError_t e = col_pass<T>(2, ia, ib, ic, id, ox, nullptr, nullptr, nullptr,
+                                      bufs[jj].d, L.n, first ? nr : L.n, first ? es : S, S, S,
+                                      L.kin, c_pad, st);
+    if (e != cudaSuccess) return (int)e;
+    launches += 1;
+  }
+  g_last_launches = launches;
+  return TRIDIAG_OK;
+}
+
+// Pass plan of tridiag_solve_batched_strided_large.  kind: 0 = no passes
+// (the on-chip strided path, m in *m), 1 = row passes (large-n plan),
+// 2 = column passes; negative = status code.
+struct StridedPlan {
+  int kind = 0;
+  int64_t m = 0, n_last = 0;
+  std::vector<LargeLevel> lv;
+};
+int strided_plan(int64_t n, int64_t S, int64_t es, int dtype, int algo, int switch_level,
+                 int64_t bottom_n, int64_t m_validated, StridedPlan* P) {
+  const int64_t np = pad_n(n);
+  P->m = m_validated;
+  const bool has_cr = algo == TRIDIAG_CR || is_hybrid(algo);
+  if (es == 1) {  // rows (contiguous or pitched): the large-n row passes
+    const int64_t bn = resolve_bottom_n(dtype, bottom_n);
+    if (bn < 0) return TRIDIAG_ERR_BOTTOM_N;
+    if (np <= bn || !has_cr) {
+      if (np > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
+      if (is_hybrid(algo) && switch_level == 0) P->m = auto_m(np, dtype, algo);
+      if (is_hybrid(algo) && P->m > tridiag_max_switch_level(dtype, algo, np)) return TRIDIAG_ERR_SWITCH_LEVEL;
+      P->kind = 0;
+      return TRIDIAG_OK;
+    }
+    P->m = large_m(np, dtype, algo, switch_level, bn);
+    if (P->m < 0) return TRIDIAG_ERR_SWITCH_LEVEL;
+    if (!large_plan(np, dtype, P->m, bn, &P->lv, &P->n_last)) return TRIDIAG_ERR_SWITCH_LEVEL;
+    P->kind = 1;
+    return TRIDIAG_OK;
+  }
+  // interleaved columns
+  const int64_t bc = resolve_col_bottom(dtype, bottom_n);
+  if (bc < 0) return TRIDIAG_ERR_BOTTOM_N;
+  if (np > bc && has_cr) {
+    const int64_t m = col_m(np, dtype, algo, switch_level, bc, &P->lv, &P->n_last);
+    if (m > 0) {
+      P->m = m;
+      P->kind = 2;
+      return TRIDIAG_OK;
+    }
+  }
+  // no pass plan (PCR / RD, an m beyond the reduced size, or n <= bottom):
+  // the on-chip strided kernels
+  if (np > tridiag_max_n(dtype, algo)) return TRIDIAG_ERR_N_TOO_LARGE;
+  if (is_hybrid(algo)) {
+    P->m = switch_level == 0 ? auto_m(np, dtype, algo) : switch_level;
+    if (P->m > tridiag_max_switch_level(dtype, algo, np)) return TRIDIAG_ERR_SWITCH_LEVEL;
+  }
+  P->kind = 0;
   return TRIDIAG_OK;
 }
 
@@ -539,11 +703,77 @@ int tridiag_solve_batched_large(const void* a, const void* b, const void* c, con
     return solve_large_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
                                 static_cast<const float*>(c), static_cast<const float*>(d),
                                 static_cast<float*>(x), n, num_systems, dtype, algo, m, lv, n_last,
-                                ws, st);
+                                ws, st, n);
   return solve_large_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
                                static_cast<const double*>(c), static_cast<const double*>(d),
                                static_cast<double*>(x), n, num_systems, dtype, algo, m, lv, n_last,
-                               ws, st);
+                               ws, st, n);
+}
+
+int64_t tridiag_column_chunk(int dtype) {
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return 0;
+  return col_chunk_n(dtype);
+}
+
+int64_t tridiag_strided_large_workspace_bytes(int64_t n, int64_t num_systems,
+                                              int64_t elem_stride, int64_t sys_stride, int dtype,
+                                              int algo, int switch_level, int64_t bottom_n) {
+  if (n < 1 || num_systems < 0 || (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64)) return -1;
+  if (algo < TRIDIAG_CR || algo > TRIDIAG_RD_STONE) return -1;
+  if (elem_stride < 1 || sys_stride < 1) return -1;
+  if (pad_n(n) > tridiag_max_n_large(dtype, algo)) return -1;
+  StridedPlan P;
+  if (strided_plan(n, num_systems, elem_stride, dtype, algo, switch_level, bottom_n, switch_level, &P) !=
+      TRIDIAG_OK)
+    return -1;
+  if (P.kind == 1) return (int64_t)large_ws_bytes(P.lv, num_systems, dtype);
+  if (P.kind == 2) return (int64_t)col_ws_bytes(P.lv, num_systems, dtype);
+  return 0;
+}
+
+int tridiag_solve_batched_strided_large(const void* a, const void* b, const void* c,
+                                        const void* d, void* x, int64_t n, int64_t num_systems,
+                                        int64_t elem_stride, int64_t sys_stride, int dtype,
+                                        int algo, int switch_level, int64_t bottom_n,
+                                        void* workspace, int64_t workspace_bytes,
+                                        tridiag_stream_t stream) {
+  g_last_launches = 0;
+  int64_t m = 0;
+  const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, elem_stride,
+                         sys_stride, true);
+  if (v != TRIDIAG_OK) return v;
+  StridedPlan P;
+  const int pv = strided_plan(n, num_systems, elem_stride, dtype, algo, switch_level, bottom_n, m, &P);
+  if (pv != TRIDIAG_OK) return pv;
+  cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+  if (P.kind == 0)
+    return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, P.m, st,
+                        Layout{elem_stride, sys_stride});
+  if (num_systems == 0) return TRIDIAG_OK;
+  const size_t need = P.kind == 1 ? large_ws_bytes(P.lv, num_systems, dtype)
+                                  : col_ws_bytes(P.lv, num_systems, dtype);
+  if (!workspace || workspace_bytes < 0 || (size_t)workspace_bytes < need) return TRIDIAG_ERR_WORKSPACE;
+  char* ws = static_cast<char*>(workspace);
+  if (P.kind == 1) {
+    if (dtype == TRIDIAG_F32)
+      return solve_large_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
+                                  static_cast<const float*>(c), static_cast<const float*>(d),
+                                  static_cast<float*>(x), n, num_systems, dtype, algo, P.m, P.lv,
+                                  P.n_last, ws, st, num_systems > 1 ? sys_stride : n);
+    return solve_large_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
+                                 static_cast<const double*>(c), static_cast<const double*>(d),
+                                 static_cast<double*>(x), n, num_systems, dtype, algo, P.m, P.lv,
+                                 P.n_last, ws, st, num_systems > 1 ? sys_stride : n);
+  }
+  if (dtype == TRIDIAG_F32)
+    return solve_col_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
+                              static_cast<const float*>(c), static_cast<const float*>(d),
+                              static_cast<float*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
+                              P.lv, P.n_last, ws, st);
+  return solve_col_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
+                             static_cast<const double*>(c), static_cast<const double*>(d),
+                             static_cast<double*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
+                             P.lv, P.n_last, ws, st);
 }
 
 // Host pipeline depth: three chunk buffers on three streams, so the

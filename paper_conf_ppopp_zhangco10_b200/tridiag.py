@@ -78,6 +78,13 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_max_n_large.restype = I64
         L.tridiag_large_chunk.argtypes = [I]
         L.tridiag_large_chunk.restype = I64
+        L.tridiag_solve_batched_strided_large.argtypes = [P, P, P, P, P, I64, I64, I64, I64, I, I,
+                                                          I, I64, P, I64, P]
+        L.tridiag_solve_batched_strided_large.restype = I
+        L.tridiag_strided_large_workspace_bytes.argtypes = [I64, I64, I64, I64, I, I, I, I64]
+        L.tridiag_strided_large_workspace_bytes.restype = I64
+        L.tridiag_column_chunk.argtypes = [I]
+        L.tridiag_column_chunk.restype = I64
         _lib = L
         return L
 
@@ -125,6 +132,20 @@ def large_workspace_bytes(n: int, num_systems: int, dtype, algo, switch_level=0,
                                                  int(bottom_n)))
     if v < 0:
         raise ValueError("tridiag: invalid arguments for the large-n path")
+    return v
+
+
+def column_chunk(dtype) -> int:
+    return int(load().tridiag_column_chunk(_dtype_code(dtype)))
+
+
+def strided_large_workspace_bytes(n: int, num_systems: int, elem_stride: int, sys_stride: int,
+                                  dtype, algo, switch_level=0, bottom_n=0) -> int:
+    v = int(load().tridiag_strided_large_workspace_bytes(
+        int(n), int(num_systems), int(elem_stride), int(sys_stride), _dtype_code(dtype),
+        _algo_code(algo), int(switch_level), int(bottom_n)))
+    if v < 0:
+        raise ValueError("tridiag: invalid arguments for the strided large path")
     return v
 
 
@@ -218,19 +239,54 @@ def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None
     ss, es = d.stride()
     if stream is None:
         stream = torch.cuda.current_stream(d.device)
-    if (_pad_n(n) > max_n(d.dtype, algo) and es == 1 and (ss == n or S <= 1)
+    contiguous = es == 1 and (ss == n or S <= 1)
+    if (_pad_n(n) > max_n(d.dtype, algo) and contiguous
             and _pad_n(n) <= max_n_large(d.dtype, algo)):
         return solve_batched_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
                                    stream=stream)
+    if not contiguous:
+        # pitched rows / interleaved columns: the workspace entry point (column
+        # or row passes where the on-chip strided kernels would be slow or
+        # too small; none needed otherwise)
+        return solve_batched_strided_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
+                                           stream=stream)
     with torch.cuda.device(d.device):
-        if es == 1 and (ss == n or S <= 1):
-            st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
-                                   x.data_ptr(), n, S, d.dtype, algo, switch_level,
-                                   stream.cuda_stream)
-        else:
-            st = solve_batched_strided_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
-                                           x.data_ptr(), n, S, es, max(ss, 1), d.dtype, algo,
-                                           switch_level, stream.cuda_stream)
+        st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                               x.data_ptr(), n, S, d.dtype, algo, switch_level,
+                               stream.cuda_stream)
+    check(st)
+    return x
+
+
+def solve_batched_strided_large(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, bottom_n=0,
+                                workspace=None, stream=None):
+    """tridiag_solve_batched_strided_large: (S, n) CUDA tensor views with
+    identical strides (pitched rows, or interleaved columns such as
+    ``grid.T``).  Interleaved systems with n > 32 R go through column CR
+    passes with a workspace (allocated from torch's caching allocator on
+    ``stream`` if None); rows beyond one CTA through the large-n row passes."""
+    if x is None:
+        x = torch.empty_strided(d.shape, d.stride(), dtype=d.dtype, device=d.device)
+    _check_tensors([a, b, c, d, x], "cuda", same_strides=True)
+    S, n = d.shape
+    ss, es = d.stride()
+    ss, es = max(ss, 1), max(es, 1)
+    if stream is None:
+        stream = torch.cuda.current_stream(d.device)
+    try:
+        need = strided_large_workspace_bytes(n, S, es, ss, d.dtype, algo, switch_level, bottom_n)
+    except ValueError:
+        need = 0  # the call itself reports the precise status
+    if workspace is None and need > 0:
+        with torch.cuda.device(d.device), torch.cuda.stream(stream):
+            workspace = torch.empty(need, dtype=torch.uint8, device=d.device)
+    wp = workspace.data_ptr() if workspace is not None else None
+    wn = workspace.numel() if workspace is not None else 0
+    with torch.cuda.device(d.device):
+        st = load().tridiag_solve_batched_strided_large(
+            a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(), x.data_ptr(), n, S, es, ss,
+            _dtype_code(d.dtype), _algo_code(algo), int(switch_level), int(bottom_n), wp, wn,
+            stream.cuda_stream)
     check(st)
     return x
 

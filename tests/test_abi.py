@@ -195,3 +195,49 @@ def test_large_n_validation():
     assert large(16384, S=0, algo=CR_PCR, m=8192) == -7    # m > max inner m
     assert large(16384, S=0, algo=CR_PCR, m=3) == -7
     assert td.status_string(-11).startswith("invalid bottom_n")
+
+
+def strided_large(n, S=4, es=None, ss=1, dtype=F32, algo=CR, m=0, bottom_n=0, ws=0x60000000,
+                  ws_bytes=1 << 40):
+    es = max(S, 64) if es is None else es
+    return int(td.load().tridiag_solve_batched_strided_large(A, B, C, D, X, n, S, es, ss, dtype,
+                                                             algo, m, bottom_n, ws, ws_bytes, None))
+
+
+def test_strided_large_workspace():
+    """Column passes (ADI column sweep, NEXT f1 + f2): 4 interleaved arrays of
+    n >> kin rows per pass level, 256-B aligned; rows (es = 1) are the large-n
+    plan; PCR / RD and n <= 32 R need none (validation only)."""
+    assert td.column_chunk(F32) == 128 and td.column_chunk(F64) == 64
+    # fp32 4096 x 4096 columns: one pass 4096 -> 256
+    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F32, CR_PCR) == 4 * 4096 * 256 * 4
+    # fp64: 4096 -> 512 -> 64 (log2 R = 3 levels per pass, bottom 32 R = 256)
+    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F64, CR) == \
+        4 * 4096 * 512 * 8 + 4 * 4096 * 64 * 8
+    S = 3  # ragged S: 256-B alignment of each array
+    assert td.strided_large_workspace_bytes(2048, S, S, 1, F32, CR) == 4 * (-(-S * 128 * 4 // 256) * 256)
+    for algo in (PCR, RD):
+        assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, algo) == 0
+    assert td.strided_large_workspace_bytes(512, 40, 40, 1, F32, CR) == 0          # on chip
+    assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, CR_PCR, 1024) == 0  # m beyond the passes
+    # rows: the large-n plan (pitched rows allowed)
+    assert td.strided_large_workspace_bytes(1 << 20, 3, 1, 1 << 20, F32, CR) == \
+        td.large_workspace_bytes(1 << 20, 3, F32, CR)
+    assert td.strided_large_workspace_bytes(8192, 3, 1, 8200, F32, CR) == 0
+    with pytest.raises(ValueError):
+        td.strided_large_workspace_bytes(4096, 40, 40, 1, F32, CR, 0, 1000)
+
+
+def test_strided_large_validation():
+    assert strided_large(4096, S=0) == 0
+    assert strided_large(4096, S=40, ws=0) == -9                 # passes need a workspace
+    assert strided_large(4096, S=40, ws_bytes=1024) == -9
+    assert strided_large(4096, S=40, bottom_n=1000) == -11        # not a power of two
+    assert strided_large(4096, S=40, bottom_n=32) == -11          # below column chunk / 2
+    assert strided_large(4096, S=40, bottom_n=1024) == -11        # above 32 R
+    assert strided_large(4096, S=0, bottom_n=64) == 0
+    assert strided_large(1 << 15, S=0) == 0                       # beyond tridiag_max_n: passes
+    assert strided_large(1 << 15, S=0, algo=PCR) == -3            # PCR has no CR levels
+    assert strided_large(4096, S=40, es=40, ss=2) == -10          # neither stride 1
+    assert strided_large(4096, S=0, algo=CR_PCR, m=3) == -7
+    assert strided_large(4096, S=0, algo=CR_PCR, m=8192) == -7
