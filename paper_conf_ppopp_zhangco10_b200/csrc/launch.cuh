@@ -60,8 +60,9 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
             : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
                                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
                   : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
-  const int occ = occupancy(dev, kern, threads,
-                            vec ? 0 : (size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T));
+  const size_t tiles = vec ? 0 : (((size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15));
+  const size_t smem = tiles + (size_t)wpb * tdg::pcr_scratch_bytes<T, R, INNER, KB>();
+  const int occ = occupancy(dev, kern, threads, smem);
   if (occ <= 0) return cudaErrorInvalidConfiguration;
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
@@ -69,7 +70,6 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
-  const size_t smem = vec ? 0 : (size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T);
   kern<<<(unsigned)grid, threads, smem, st>>>(a, b, c, d, x, (int)n, (long long)S, k, log2P,
                                            vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
                                            (long long)L.ss, stamps);

@@ -148,6 +148,9 @@ tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __r
   const int G = Gm.G(), P = Gm.P();
   const int TE = ilv_tile_elems(P * R, G);
   T* tX = tile + 4 * TE;
+  // (the tiles leave no room for the cyclic PCR relayout's scratch: the
+  // block-layout PCR with shuffles runs here)
+  T* pcr_scr = nullptr;
   const int g = threadIdx.x >> Gm.lp;
   const int ls = threadIdx.x & (P - 1);
   // lane-blocked rows ls R + q of system g: offset base + q G (R | 16 or 16 | R)
@@ -169,7 +172,7 @@ tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __r
     if (tn < tiles) ilv_issue<T, R, LP, true>(a, b, c, d, tile, TE, tn * G, S, 0, n_real, es, Gm, c_pad);
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
-    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P);
+    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, Stamp(), pcr_scr);
 #pragma unroll
     for (int q = 0; q < R; ++q) tX[base + q * G] = rd[q];
     __syncthreads();

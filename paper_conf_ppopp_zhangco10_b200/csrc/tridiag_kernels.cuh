@@ -45,7 +45,8 @@ struct Stamp {
 // KB >= 0: k == KB < LR (m = P * (R >> KB) > P, register-blocked inner solve).
 template <typename T, int R, int INNER, int KB>
 __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&d)[R], int k,
-                                           int ls, int P, Stamp st = Stamp()) {
+                                           int ls, int P, Stamp st = Stamp(),
+                                           T* pcr_scratch = nullptr) {
   constexpr int LR = ilog2c(R);
   constexpr int kin = KB < 0 ? LR : KB;
   inlane_forward_interior<T, R>(a, b, c, d, kin);
@@ -62,7 +63,7 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
   } else {
     // m = P * (R >> KB) > P: the intermediate system stays block-distributed
     // in registers (no copy; the paper copies it to 5 extra arrays).
-    if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
+    if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P, pcr_scratch);
     else blocked_rd<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
   }
   st.mark(3);
@@ -160,6 +161,13 @@ __device__ __forceinline__ void warp_kernel_body(
   const int sub = lane >> log2P;
   const int ls = lane & (P - 1);
   const long long step = (long long)gridDim.x * wpb * G;
+  // per-warp scratch of the cyclic PCR relayout, after the GEN warp tiles
+  T* pcr_scr = nullptr;
+  if constexpr (pcr_scratch_bytes<T, R, INNER, KB>() > 0) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    const size_t off = GEN ? (((size_t)wpb * 4 * warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15)) : 0;
+    pcr_scr = reinterpret_cast<T*>(smem_raw + off + (size_t)warp * pcr_scratch_bytes<T, R, INNER, KB>());
+  }
   int iter = 0;
   for (long long s0 = ((long long)blockIdx.x * wpb + warp) * G; s0 < S; s0 += step, ++iter) {
     Stamp stp;
@@ -199,7 +207,7 @@ __device__ __forceinline__ void warp_kernel_body(
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
-    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp);
+    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp, pcr_scr);
     if constexpr (!GEN) {
       if (valid) store_block<T, R>(x + off, rd, vec);
     } else {
