@@ -27,6 +27,11 @@ CASES = [
     (torch.float32, 1000, 7, "rd", 0, "contig"),         # CTA-blocked RD, staged ragged path
     (torch.float32, 16384, 2, "cr_pcr", 0, "contig"),    # large-n passes
     (torch.float64, 12289, 2, "cr_rd", 0, "contig"),     # large-n passes, ragged, RD inner
+    (torch.float32, 256, 40, "pcr", 0, "contig"),        # cyclic PCR relayout, 2 systems / warp
+    (torch.float64, 256, 40, "pcr", 0, "contig"),        # same, fp64 slots
+    (torch.float32, 2048, 64, "cr_pcr", 0, "column"),    # column passes, TMA-fed
+    (torch.float32, 1000, 37, "cr_pcr", 0, "column"),    # column passes, direct loads, ragged
+    (torch.float64, 2048, 40, "cr", 0, "column"),        # column passes fp64, two levels
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
