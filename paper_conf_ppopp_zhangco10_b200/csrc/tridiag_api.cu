@@ -461,11 +461,51 @@ size_t col_ws_bytes(const std::vector<LargeLevel>& lv, int64_t S, int dtype) {
   return total;
 }
 
+// Pass plan of tridiag_solve_batched_strided_large.  kind: 0 = no passes
+// (the on-chip strided path, m in *m), 1 = row passes (large-n plan),
+// 2 = column passes; negative = status code.
+struct StridedPlan {
+  int kind = 0;
+  int64_t m = 0, n_last = 0;
+  std::vector<LargeLevel> lv;
+};
+
+// The single-pass column kernel (tridiag_colfused.cuh) replaces the passes
+// when the caller leaves bottom_n at its default and the shape allows it.
+bool col_fused_ok(int64_t np, int dtype, int algo, int64_t m, int64_t bottom_n) {
+  if (bottom_n != 0) return false;
+  const int inner = algo == TRIDIAG_CR_RD ? tdg::kRD : tdg::kPCR;
+  return dtype == TRIDIAG_F64 ? col_fused_eligible<double>(np, inner, m)
+                              : col_fused_eligible<float>(np, inner, m);
+}
+
+// Workspace of a column plan: the passes' levels, or the fused kernel's
+// survivors + counters if that is larger (either may run: the fused kernel
+// needs TMA-describable pointers, known only at the call).
+size_t col_need(const StridedPlan& P, int64_t n, int64_t S, int dtype, int algo, int64_t bottom_n) {
+  size_t need = col_ws_bytes(P.lv, S, dtype);
+  const int64_t np = pad_n(n);
+  if (col_fused_ok(np, dtype, algo, P.m, bottom_n)) {
+    const size_t f = dtype == TRIDIAG_F64 ? col_fused_ws_bytes<double>(np, S) : col_fused_ws_bytes<float>(np, S);
+    need = std::max(need, f);
+  }
+  return need;
+}
+
 template <typename T>
 int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
                 int64_t es, int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
-                int64_t n_last, char* ws, cudaStream_t st) {
+                int64_t n_last, char* ws, cudaStream_t st, bool fused) {
   const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
+  if (fused) {
+    cudaError_t e = cudaSuccess;
+    const int inner = algo == TRIDIAG_CR_RD ? tdg::kRD : tdg::kPCR;
+    if (col_fused<T>(a, b, c, d, x, pad_n(nr), nr, es, S, inner, m, c_pad, ws, st, &e)) {
+      if (e != cudaSuccess) return (int)e;
+      g_last_launches = 1;
+      return TRIDIAG_OK;
+    }
+  }
   struct Buf { T* a; T* b; T* c; T* d; };
   std::vector<Buf> bufs;
   char* p = ws;
@@ -513,14 +553,6 @@ int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr
   return TRIDIAG_OK;
 }
 
-// Pass plan of tridiag_solve_batched_strided_large.  kind: 0 = no passes
-// (the on-chip strided path, m in *m), 1 = row passes (large-n plan),
-// 2 = column passes; negative = status code.
-struct StridedPlan {
-  int kind = 0;
-  int64_t m = 0, n_last = 0;
-  std::vector<LargeLevel> lv;
-};
 int strided_plan(int64_t n, int64_t S, int64_t es, int dtype, int algo, int switch_level,
                  int64_t bottom_n, int64_t m_validated, StridedPlan* P) {
   const int64_t np = pad_n(n);
@@ -727,7 +759,7 @@ int64_t tridiag_strided_large_workspace_bytes(int64_t n, int64_t num_systems,
       TRIDIAG_OK)
     return -1;
   if (P.kind == 1) return (int64_t)large_ws_bytes(P.lv, num_systems, dtype);
-  if (P.kind == 2) return (int64_t)col_ws_bytes(P.lv, num_systems, dtype);
+  if (P.kind == 2) return (int64_t)col_need(P, n, num_systems, dtype, algo, bottom_n);
   return 0;
 }
 
@@ -751,7 +783,7 @@ int tridiag_solve_batched_strided_large(const void* a, const void* b, const void
                         Layout{elem_stride, sys_stride});
   if (num_systems == 0) return TRIDIAG_OK;
   const size_t need = P.kind == 1 ? large_ws_bytes(P.lv, num_systems, dtype)
-                                  : col_ws_bytes(P.lv, num_systems, dtype);
+                                  : col_need(P, n, num_systems, dtype, algo, bottom_n);
   if (!workspace || workspace_bytes < 0 || (size_t)workspace_bytes < need) return TRIDIAG_ERR_WORKSPACE;
   char* ws = static_cast<char*>(workspace);
   if (P.kind == 1) {
@@ -765,15 +797,16 @@ int tridiag_solve_batched_strided_large(const void* a, const void* b, const void
                                  static_cast<double*>(x), n, num_systems, dtype, algo, P.m, P.lv,
                                  P.n_last, ws, st, num_systems > 1 ? sys_stride : n);
   }
+  const bool fused = col_fused_ok(pad_n(n), dtype, algo, P.m, bottom_n);
   if (dtype == TRIDIAG_F32)
     return solve_col_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
                               static_cast<const float*>(c), static_cast<const float*>(d),
                               static_cast<float*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
-                              P.lv, P.n_last, ws, st);
+                              P.lv, P.n_last, ws, st, fused);
   return solve_col_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
                              static_cast<const double*>(c), static_cast<const double*>(d),
                              static_cast<double*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
-                             P.lv, P.n_last, ws, st);
+                             P.lv, P.n_last, ws, st, fused);
 }
 
 // Host pipeline depth: three chunk buffers on three streams, so the

@@ -172,3 +172,58 @@ def test_column_sweep_of_a_grid_full_size_sampled():
     idx = torch.randperm(S, generator=torch.Generator().manual_seed(0))[:64].tolist()
     sub = [t[idx] for t in rows]
     assert err(*sub, x[idx]).max() <= TOL[torch.float32]
+
+
+# ---------------------------------------------------------------------------
+# Single-pass column kernel (tridiag_colfused.cuh): one launch, the same CR
+# levels in the same correctly rounded operations as the passes and the
+# contiguous kernels, so bitwise equal to both.
+# ---------------------------------------------------------------------------
+FUSED_N = {torch.float32: (1024, 2048, 4096, 8192), torch.float64: (512, 1024, 2048, 4096)}
+
+
+def _passes(monkeypatch, on):
+    monkeypatch.setenv("TRIDIAG_COL_FUSED", "1" if on else "0")
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_column_fused_bitwise(dtype, monkeypatch):
+    for n in FUSED_N[dtype]:
+        for S in (36, 96):  # row pitch a multiple of 16 B (TMA)
+            rows = gen("dd", S, n, dtype, seed=n * 7 + S)
+            views = as_columns(rows)
+            for algo, m in (("cr", 0), ("cr_pcr", 0), ("cr_pcr", 2), ("cr_pcr", 8), ("cr_pcr", 32)):
+                ref = td.solve_batched(*rows, algo=algo, switch_level=m)
+                _passes(monkeypatch, True)
+                x = cols_solve(views, algo, m)
+                assert td.last_launch_count() == 1, (n, S, algo, m)
+                assert torch.equal(x.contiguous(), ref), (n, S, algo, m,
+                                                          (x.contiguous() - ref).abs().max().item())
+                _passes(monkeypatch, False)
+                xp = cols_solve(views, algo, m)
+                assert td.last_launch_count() > 1
+                assert torch.equal(xp, x)
+            assert err(*rows, x).max() <= TOL[dtype], (n, S)
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_column_fused_ragged_in_place_cr_rd(dtype, monkeypatch):
+    _passes(monkeypatch, True)
+    nmax = FUSED_N[dtype][-1]
+    for n, S in ((nmax - 96, 44), (FUSED_N[dtype][0] + 1, 8), (FUSED_N[dtype][1] - 5, 64)):
+        rows = gen("dd", S, n, dtype, seed=n)
+        views = as_columns(rows)
+        ref = td.solve_batched(*rows, algo="cr_pcr")
+        dcol = views[3]
+        keep = views[0].clone()
+        cols_solve(views[:3] + [dcol], "cr_pcr", x=dcol)
+        assert td.last_launch_count() == 1, n
+        assert torch.equal(dcol.contiguous(), ref), n
+        assert torch.equal(views[0], keep)
+    n = FUSED_N[dtype][2]
+    rows = gen("rdw", 40, n, dtype, seed=9)
+    views = as_columns(rows)
+    for m in (0, 8, 32):
+        x = cols_solve(views, "cr_rd", m)
+        assert td.last_launch_count() == 1, m
+        assert err(*rows, x).max() <= TOL[dtype], m
