@@ -32,6 +32,8 @@ CASES = [
     (torch.float32, 2048, 64, "cr_pcr", 0, "column"),    # column passes, TMA-fed
     (torch.float32, 1000, 37, "cr_pcr", 0, "column"),    # column passes, direct loads, ragged
     (torch.float64, 2048, 40, "cr", 0, "column"),        # column passes fp64, two levels
+    (torch.float32, 2048, 64, "cr_pcr", 0, "column_fused"),  # single-kernel column sweep
+    (torch.float64, 1000, 40, "cr_rd", 0, "column_fused"),   # same, fp64, ragged n, RD inner
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
@@ -41,12 +43,15 @@ for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
         continue
     fam = "rdw" if algo in ("rd", "cr_rd") else "dd"
     a, b, c, d = inputs.generate(fam, S, n, dt, device="cuda")
-    if layout == "column":
+    os.environ["TRIDIAG_COL_FUSED"] = "1" if layout == "column_fused" else "0"
+    if layout in ("column", "column_fused"):
         views = [t.t().contiguous().t() for t in (a, b, c, d)]
     else:
         views = [a, b, c, d]
     x = td.solve_batched(*views, algo=algo, switch_level=m)
     torch.cuda.synchronize()
+    if layout == "column_fused":
+        assert td.last_launch_count() == 1, "single-kernel path did not run"
     ref = oracle.thomas(*[t.cpu().numpy() for t in (a, b, c, d)])
     e = float(np.max(oracle.normwise_error(x.contiguous().cpu().numpy(), ref)))
     tol = 1e-4 if dt == torch.float32 else 1e-10
