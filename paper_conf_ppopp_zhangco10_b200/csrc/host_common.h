@@ -12,6 +12,7 @@
 #include <map>
 #include <mutex>
 #include <tuple>
+#include <utility>
 
 #include "tridiag.h"
 
@@ -39,6 +40,29 @@ int blocked_minb();
 // diagnostic only: the one device allocation the library ever makes).
 long long* stamp_buffer(int64_t elems);
 PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
+
+// Programmatic dependent launch (TRIDIAG_PDL, default 1): see pdl_entry().
+int pdl_mode();
+
+// Launch with the programmatic-stream-serialization attribute (when enabled):
+// the kernel's CTAs may be scheduled while the previous grid on the stream
+// drains; every kernel of the library starts with pdl_entry(), which waits
+// for that grid before touching global memory.
+template <typename... KArgs, typename... Args>
+cudaError_t launch_k(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t st,
+                     Args&&... args) {
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = grid;
+  cfg.blockDim = block;
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = st;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[0].val.programmaticStreamSerializationAllowed = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = pdl_mode() ? 1 : 0;
+  return cudaLaunchKernelEx(&cfg, kern, std::forward<Args>(args)...);
+}
 
 std::mutex& occ_mutex();
 std::map<std::tuple<int, const void*, int, size_t>, int>& occ_cache();

@@ -85,6 +85,12 @@ int prefetch_mode() {
   if (v < 0) v = env_int("TRIDIAG_PREFETCH", 2);
   return v;
 }
+int pdl_mode() {
+  static int v = -1;
+  if (v < 0) v = env_int("TRIDIAG_PDL", 1);
+  return v;
+}
+
 int tma_mode() {
   static int v = env_int("TRIDIAG_TMA", 1);
   return v;

@@ -130,6 +130,7 @@ tdg_col_fused_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_const
                      const __grid_constant__ CUtensorMap teC, const __grid_constant__ CUtensorMap teD,
                      T* x, T* ws, unsigned* cnt, long long n, long long n_real, long long es,
                      long long S, int k2, T c_pad, int nf) {
+  pdl_entry();
   constexpr int LR = ilog2c(R);
   constexpr int HE = col_heads_elems<T, R>();
   constexpr long long CH = (long long)W * R;

@@ -105,6 +105,7 @@ tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
                       const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                       T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
                       long long es, long long S, long long es2, T c_pad) {
+  pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -169,6 +170,7 @@ __global__ void __launch_bounds__(W * 32, 2)
 tdg_col_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                       const T* d, T* x, const T* __restrict__ x2, long long n, long long n_real,
                       long long es, long long S, long long es2, T c_pad) {
+  pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
@@ -267,6 +269,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                           T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
                           long long es, long long S, long long es2, T c_pad) {
+  pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -352,6 +355,7 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
                           T* x, const T* __restrict__ x2, long long n, long long n_real,
                           long long es, long long S, long long es2, T c_pad) {
+  pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
   constexpr uint32_t ARR = col_stage_bytes<T, R, W>() / 4;

@@ -224,6 +224,7 @@ __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                 int n_real, T c_pad, long long es, long long ss, long long* stamps) {
+  pdl_entry();
   warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
                                          es, ss, stamps);
 }
@@ -237,6 +238,7 @@ __global__ void __launch_bounds__(256, (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
+  pdl_entry();
   warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
                                          es, ss, stamps);
 }
@@ -523,6 +525,7 @@ __global__ void __launch_bounds__(W * 32)
 tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                const T* d, T* x, int n, long long S, int k, int vec, int pf, int n_real,
                T c_pad, long long es, long long ss) {
+  pdl_entry();
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;

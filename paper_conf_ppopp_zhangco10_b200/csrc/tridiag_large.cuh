@@ -68,6 +68,7 @@ __global__ void __launch_bounds__(128)
 tdg_large_heads_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                        const T* __restrict__ d, T* __restrict__ hbuf, long long n, long long n_real,
                        long long ss, long long S, int chunk, int vec, T c_pad) {
+  pdl_entry();
   constexpr int NH = large_heads_elems<R>() / 4;
   const long long C = n / chunk;
   const long long total = S * (C - 1);
@@ -141,6 +142,7 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
                         const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                         T* __restrict__ c2, T* __restrict__ d2, const T* __restrict__ hbuf,
                         long long n, long long n_real, long long ss, long long S, int vec, T c_pad) {
+  pdl_entry();
   constexpr int P = 32 * W;
   constexpr int NH = large_heads_elems<R>() / 4;
   constexpr int Q = R >> KIN;
@@ -175,6 +177,7 @@ __global__ void __launch_bounds__(W * 32)
 tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, const T* __restrict__ x2, const T* __restrict__ hbuf,
                         long long n, long long n_real, long long ss, long long S, int vec, T c_pad) {
+  pdl_entry();
   constexpr int P = 32 * W;
   constexpr int NH = large_heads_elems<R>() / 4;
   constexpr int Q = R >> KIN;
