@@ -471,3 +471,39 @@ def test_full_size_bench_config_sampled():
     idx = torch.randperm(S, generator=torch.Generator().manual_seed(0))[:512].cuda()
     e = err_vs_oracle(a[idx], b[idx], c[idx], d[idx], x[idx])
     assert e.max() <= 1e-4
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_dependent_launch_chain_adi(dtype):
+    """Launches carry the programmatic-dependent-launch attribute: each kernel
+    waits (griddepcontrol.wait) for the previous grid before its first global
+    access.  An ADI-like chain with no host synchronisation -- row sweep,
+    column sweep of its output, row sweep again, each consuming the previous
+    x as its right-hand side -- must equal the same chain with a device
+    synchronisation after every call, bitwise, for every kernel family on the
+    path (warp, TMA CTA, interleaved tile, column passes)."""
+    for N in (512, 4096 if dtype == torch.float32 else 2048):
+        a, b, c, d = gen("dd", N, N, dtype, seed=N + 17)
+        cols = [t.t().contiguous().t() for t in (a, b, c)]
+
+        def chain(sync):
+            x1 = td.solve_batched(a, b, c, d, algo="cr_pcr")
+            if sync:
+                torch.cuda.synchronize()
+            d2 = x1.t().contiguous().t()  # the row sweep's output as column right-hand sides
+            x2 = td.solve_batched(*cols, d2, algo="cr_pcr")
+            if sync:
+                torch.cuda.synchronize()
+            x3 = td.solve_batched(a, b, c, x2.contiguous(), algo="cr")
+            if sync:
+                torch.cuda.synchronize()
+            # in place: x == d, consumed right away by the next launch
+            td.solve_batched(a, b, c, x3, x=x3, algo="cr_pcr")
+            return td.solve_batched(a, b, c, x3, algo="cr_pcr")
+
+        ref = chain(True)
+        torch.cuda.synchronize()
+        for _ in range(3):
+            out = chain(False)
+            torch.cuda.synchronize()
+            assert torch.equal(out, ref), N
