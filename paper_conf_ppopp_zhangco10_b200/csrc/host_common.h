@@ -43,6 +43,8 @@ PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 
 // Programmatic dependent launch (TRIDIAG_PDL, default 1): see pdl_entry().
 int pdl_mode();
+// Double-buffered CTA-kernel regions (TRIDIAG_CTA_DBUF, default 1).
+int cta_dbuf_mode();
 
 // Launch with the programmatic-stream-serialization attribute (when enabled):
 // the kernel's CTAs may be scheduled while the previous grid on the stream

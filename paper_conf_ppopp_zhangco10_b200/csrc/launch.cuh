@@ -143,10 +143,21 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
       }
     }
   }
-  const int occ = occupancy(dev, kern, W * 32, smem);
+  int occ = occupancy(dev, kern, W * 32, smem);
   if (occ <= 0) return cudaSuccess;
+  // double-buffered heads / survivor regions (no end-of-system barrier) when
+  // that does not cost occupancy (TRIDIAG_CTA_DBUF=0 disables)
+  size_t smem_use = smem;
+  int dbuf = 0;
+  if (cta_dbuf_mode()) {
+    const size_t smem2 = tdg::cta_tma_smem_bytes<T>(R, W, INNER, k, 2);
+    if (smem2 <= 227 * 1024 && occupancy(dev, kern, W * 32, smem2) >= occ) {
+      smem_use = smem2;
+      dbuf = (int)(tdg::cta_tma_region_bytes<T>(R, W, INNER, k) / sizeof(T));
+    }
+  }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem, st, mA, mB, mC, mD, x, (int)n, (long long)S, k); if (le_ != cudaSuccess) return le_; }
+  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf); if (le_ != cudaSuccess) return le_; }
   g_last_launches = 1;
   *used = true;
   return cudaGetLastError();

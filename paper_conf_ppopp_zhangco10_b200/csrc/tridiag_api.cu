@@ -85,6 +85,11 @@ int prefetch_mode() {
   if (v < 0) v = env_int("TRIDIAG_PREFETCH", 2);
   return v;
 }
+int cta_dbuf_mode() {
+  static int v = -1;
+  if (v < 0) v = env_int("TRIDIAG_CTA_DBUF", 1);
+  return v;
+}
 int pdl_mode() {
   static int v = -1;
   if (v < 0) v = env_int("TRIDIAG_PDL", 1);

@@ -80,7 +80,7 @@ template <typename T, int R, int W, int INNER, int KB>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
-                   T* x, int n, long long S, int k) {
+                   T* x, int n, long long S, int k, int dbuf) {
   pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
@@ -92,7 +92,7 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
   extern __shared__ __align__(1024) unsigned char smem_raw[];
   unsigned char* stage = smem_raw;
   uint64_t* bar = reinterpret_cast<uint64_t*>(smem_raw + STAGE);
-  T* heads = reinterpret_cast<T*>(smem_raw + STAGE + 16);
+  T* heads0 = reinterpret_cast<T*>(smem_raw + STAGE + 16);
   const int ls = threadIdx.x;
 
   const CUtensorMap* maps[4] = {&tmA, &tmB, &tmC, &tmD};
@@ -112,7 +112,13 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
   __syncthreads();
 
   uint32_t parity = 0;
-  for (long long sys = blockIdx.x; sys < S; sys += gridDim.x) {
+  int it = 0;
+  for (long long sys = blockIdx.x; sys < S; sys += gridDim.x, ++it) {
+    // dbuf > 0: the heads / survivor regions alternate between two copies of
+    // dbuf elements by system parity, so the next system's writes cannot
+    // race this system's reads (they are separated by the next system's
+    // first barrier) and no barrier is needed at the end of a system
+    T* heads = heads0 + ((dbuf > 0 && (it & 1)) ? dbuf : 0);
     mbar_wait(bar, parity);
     parity ^= 1;
     T ra[R], rb[R], rc[R], rd[R];
@@ -137,15 +143,20 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     }
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
     store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
-    __syncthreads();  // heads / survivor regions are reused by the next system
+    if (dbuf == 0) __syncthreads();  // heads / survivor regions are reused by the next system
   }
 }
 
 // Dynamic shared memory of tdg_cta_tma_kernel: stage + mbarrier + the
 // register path's regions (heads, lane heads, survivors, inner).
+// copies = 2: double-buffered regions (the kernel's dbuf), each rounded to 16 B.
 template <typename T>
-inline size_t cta_tma_smem_bytes(int R, int W, int inner, int k) {
-  return tma_stage_bytes<T>(R, W) + 16 + cta_smem_bytes<T>(R, W, inner, k);
+inline size_t cta_tma_region_bytes(int R, int W, int inner, int k) {
+  return (cta_smem_bytes<T>(R, W, inner, k) + 15) & ~size_t(15);
+}
+template <typename T>
+inline size_t cta_tma_smem_bytes(int R, int W, int inner, int k, int copies = 1) {
+  return tma_stage_bytes<T>(R, W) + 16 + copies * cta_tma_region_bytes<T>(R, W, inner, k);
 }
 
 }  // namespace tdg
