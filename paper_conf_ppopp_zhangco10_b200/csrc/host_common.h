@@ -45,6 +45,8 @@ PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 int pdl_mode();
 // Double-buffered CTA-kernel regions (TRIDIAG_CTA_DBUF, default 1).
 int cta_dbuf_mode();
+// 2-CTA cluster kernel for 16-warp systems (opt-in TRIDIAG_CTA_CLUSTER=1).
+int cta_cluster_mode();
 
 // Launch with the programmatic-stream-serialization attribute (when enabled):
 // the kernel's CTAs may be scheduled while the previous grid on the stream

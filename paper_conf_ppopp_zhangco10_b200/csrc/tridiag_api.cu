@@ -85,6 +85,7 @@ int prefetch_mode() {
   if (v < 0) v = env_int("TRIDIAG_PREFETCH", 2);
   return v;
 }
+int cta_cluster_mode() { return env_int("TRIDIAG_CTA_CLUSTER", 0); }  // opt-in; read per call (A/B tests)
 int cta_dbuf_mode() {
   static int v = -1;
   if (v < 0) v = env_int("TRIDIAG_CTA_DBUF", 1);

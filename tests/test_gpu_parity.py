@@ -507,3 +507,23 @@ def test_dependent_launch_chain_adi(dtype):
             out = chain(False)
             torch.cuda.synchronize()
             assert torch.equal(out, ref), N
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_cluster_kernel_bitwise_equal_single_cta(dtype, monkeypatch):
+    """The opt-in 2-CTA cluster kernel for the largest on-chip systems (fp32
+    n = 8192, fp64 n = 4096; TRIDIAG_CTA_CLUSTER=1, tridiag_cta2.cuh): the
+    same CR / inner operations as the single 16-warp CTA kernel, so bitwise
+    the same x; and within the gates."""
+    n = td.max_n(dtype, "cr")
+    for S, algo, m, fam in ((37, "cr", 0, "dd"), (300, "cr_pcr", 0, "dd"), (64, "cr_pcr", 2, "dd"),
+                            (64, "cr_pcr", 16, "dd"), (64, "cr_pcr", 32, "dd"), (40, "cr_rd", 8, "rdw"),
+                            (40, "cr_rd", 32, "rdw")):
+        a, b, c, d = gen(fam, S, n, dtype, seed=S + m)
+        monkeypatch.setenv("TRIDIAG_CTA_CLUSTER", "1")
+        x1 = gpu_solve(a, b, c, d, algo, m)
+        monkeypatch.setenv("TRIDIAG_CTA_CLUSTER", "0")
+        x0 = gpu_solve(a, b, c, d, algo, m)
+        assert torch.equal(x1, x0), (S, algo, m, (x1 - x0).abs().max().item())
+        assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (S, algo, m)
+    monkeypatch.delenv("TRIDIAG_CTA_CLUSTER")
