@@ -158,7 +158,7 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
     }
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf); if (le_ != cudaSuccess) return le_; }
+  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode()); if (le_ != cudaSuccess) return le_; }
   g_last_launches = 1;
   *used = true;
   return cudaGetLastError();

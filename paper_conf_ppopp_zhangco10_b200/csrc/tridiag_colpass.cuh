@@ -33,6 +33,13 @@
 
 #include "tridiag_tma.cuh"  // mbarrier / cp.async.bulk.tensor helpers
 
+// CTAs per SM the TMA expansion pass asks for: its 64 KB stage allows 3, which
+// caps registers at 80 -- a gain for fp64 (255 vs 267 us at 4096^2), a loss
+// for fp32 (61 vs 59 us per pass), so fp32 keeps 2.
+#ifndef TDG_COL_EXPAND_MINB
+#define TDG_COL_EXPAND_MINB(T) (sizeof(T) == 8 ? 3 : 2)
+#endif
+
 namespace tdg {
 
 // R rows of one array of column s, rows >= n_real padded (reading R26) and
@@ -268,7 +275,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                           const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                           T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
-                          long long es, long long S, long long es2, T c_pad) {
+                          long long es, long long S, long long es2, T c_pad, int pf) {
   pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
@@ -290,6 +297,11 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     mbar_arrive_expect_tx(bar, 4 * ARR);
 #pragma unroll
     for (int q = 0; q < 4; ++q) tma_load_2d(stage + q * ARR, maps[q], (int)(gg * 32), (int)(cc * CH), bar);
+    if (pf && uu - 1 >= lo) {  // the unit after: toward L2
+      const long long g2 = (uu - 1) / C, c2 = (uu - 1) - g2 * C;
+#pragma unroll
+      for (int q = 0; q < 4; ++q) tma_prefetch_2d(maps[q], (int)(g2 * 32), (int)(c2 * CH));
+    }
   };
   if (threadIdx.x == 0) {
     mbar_init(bar, 1);
@@ -350,11 +362,11 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
 }
 
 template <typename T, int R, int W, int KIN>
-__global__ void __launch_bounds__(W * 32, 2)
+__global__ void __launch_bounds__(W * 32, TDG_COL_EXPAND_MINB(T))
 tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                           const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
                           T* x, const T* __restrict__ x2, long long n, long long n_real,
-                          long long es, long long S, long long es2, T c_pad) {
+                          long long es, long long S, long long es2, T c_pad, int pf) {
   pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -371,6 +383,11 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     mbar_arrive_expect_tx(bar, 4 * ARR);
 #pragma unroll
     for (int q = 0; q < 4; ++q) tma_load_2d(stage + q * ARR, maps[q], (int)(gg * 32), (int)(cc * CH), bar);
+    if (pf && uu + gridDim.x < U) {  // the unit after: toward L2
+      const long long u2 = uu + gridDim.x, g2 = u2 / C, c2 = u2 - g2 * C;
+#pragma unroll
+      for (int q = 0; q < 4; ++q) tma_prefetch_2d(maps[q], (int)(g2 * 32), (int)(c2 * CH));
+    }
   };
   if (threadIdx.x == 0) {
     mbar_init(bar, 1);

@@ -50,6 +50,16 @@ __device__ __forceinline__ void tma_load_2d(void* dst, const CUtensorMap* map, i
       : "memory");
 }
 
+// L2 prefetch of a TMA box (no shared memory, no completion): issued for the
+// unit after the one being copied, it keeps two units per CTA in flight to
+// HBM while the stage holds only one.
+__device__ __forceinline__ void tma_prefetch_2d(const CUtensorMap* map, int c0, int c1) {
+  asm volatile("cp.async.bulk.prefetch.tensor.2d.L2.global.tile [%0, {%1, %2}];" ::"l"(
+                   reinterpret_cast<uint64_t>(map)),
+               "r"(c0), "r"(c1)
+               : "memory");
+}
+
 // One lane's 64-byte row out of the 64B-swizzled stage: 16-byte chunk ch is
 // stored at chunk ch ^ sw, sw = (row >> 1) & 3 (CU_TENSOR_MAP_SWIZZLE_64B).
 template <typename T, int R>
@@ -80,7 +90,7 @@ template <typename T, int R, int W, int INNER, int KB>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
-                   T* x, int n, long long S, int k, int dbuf) {
+                   T* x, int n, long long S, int k, int dbuf, int pf) {
   pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
@@ -104,6 +114,13 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
       for (int bx = 0; bx < NBOX; ++bx)
         tma_load_2d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0,
                     (int)(sys * P + bx * ROWS), bar);
+    if (pf && sys + gridDim.x < S) {
+#pragma unroll
+      for (int q = 0; q < 4; ++q)
+#pragma unroll
+        for (int bx = 0; bx < NBOX; ++bx)
+          tma_prefetch_2d(maps[q], 0, (int)((sys + gridDim.x) * P + bx * ROWS));
+    }
   };
   if (ls == 0) {
     mbar_init(bar, 1);
