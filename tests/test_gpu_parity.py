@@ -527,3 +527,37 @@ def test_cluster_kernel_bitwise_equal_single_cta(dtype, monkeypatch):
         assert torch.equal(x1, x0), (S, algo, m, (x1 - x0).abs().max().item())
         assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (S, algo, m)
     monkeypatch.delenv("TRIDIAG_CTA_CLUSTER")
+
+
+def _residual_rel(a, b, c, d, x):
+    a64, b64, c64, d64, x64 = (t.double() for t in (a, b, c, d, x))
+    r = b64 * x64 - d64
+    r[:, 1:] += a64[:, 1:] * x64[:, :-1]
+    r[:, :-1] += c64[:, :-1] * x64[:, 1:]
+    return r.abs().amax(dim=1) / d64.abs().amax(dim=1)
+
+
+@pytest.mark.parametrize("name,dtype,S,n,algo,fam,res_tol,samples", [
+    ("C3 rows fp32", torch.float32, 4096, 4096, "cr_pcr", "dd", 1e-5, 48),
+    ("C3 rows fp64", torch.float64, 4096, 4096, "cr_pcr", "dd", 1e-12, 48),
+    # rdw (RD-stable, not diagonally dominant: |b| ~ |c|): the residual bound
+    # is looser than DD's; the normwise error gate is the same
+    ("C3 rows RD (rdw)", torch.float32, 4096, 4096, "rd", "rdw", 5e-3, 48),
+    ("C4 2^20 x 256 fp32", torch.float32, 1 << 20, 256, "cr_pcr", "dd", 1e-5, 256),
+    ("C5 16384 x 8192 fp32", torch.float32, 16384, 8192, "cr_pcr", "dd", 1e-5, 24),
+    ("C5 16384 x 8192 fp32 CR+RD (rdw)", torch.float32, 16384, 8192, "cr_rd", "rdw", 5e-3, 24),
+])
+def test_full_size_other_configs_sampled(name, dtype, S, n, algo, fam, res_tol, samples):
+    """The other BASELINE.json configs at their full sizes, in the launch
+    configuration bench.py times (one call, tuned m): every system's relative
+    residual ||Ax - d||_inf / ||d||_inf (a property at any size, fp64 torch
+    ops), and sampled systems vs the fp64 oracle within the gate."""
+    a, b, c, d = gen(fam, S, n, dtype, seed=20100109 + n)
+    x = gpu_solve(a, b, c, d, algo)
+    assert torch.isfinite(x).all(), name
+    rel = torch.cat([_residual_rel(a[i:i + 8192], b[i:i + 8192], c[i:i + 8192], d[i:i + 8192],
+                                   x[i:i + 8192]) for i in range(0, S, 8192)])
+    assert float(rel.max()) <= res_tol, (name, float(rel.max()))
+    idx = torch.randperm(S, generator=torch.Generator().manual_seed(1))[:samples].cuda()
+    e = err_vs_oracle(a[idx], b[idx], c[idx], d[idx], x[idx])
+    assert e.max() <= TOL[dtype], (name, e.max())
