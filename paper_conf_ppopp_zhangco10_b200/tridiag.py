@@ -113,8 +113,26 @@ def check(status: int) -> None:
         raise TridiagError(f"tridiag: CUDA error {status}: {status_string(status)}")
 
 
+_MAX_N = {}  # (dtype code, algo code) -> tridiag_max_n (immutable per build)
+
+# torch's own fast accessors (what torch.cuda.current_stream / current_device
+# call underneath), with the public API as the fallback
+_current_device = getattr(torch._C, "_cuda_getDevice", None) or torch.cuda.current_device
+_raw_stream = getattr(torch._C, "_cuda_getCurrentRawStream", None)
+
+
+def _current_raw_stream(index: int) -> int:
+    if _raw_stream is not None:
+        return _raw_stream(index)
+    return torch.cuda.current_stream(index).cuda_stream
+
+
 def max_n(dtype, algo) -> int:
-    return int(load().tridiag_max_n(_dtype_code(dtype), _algo_code(algo)))
+    key = (_dtype_code(dtype), _algo_code(algo))
+    v = _MAX_N.get(key)
+    if v is None:
+        v = _MAX_N[key] = int(load().tridiag_max_n(*key))
+    return v
 
 
 def max_n_large(dtype, algo) -> int:
@@ -150,10 +168,7 @@ def strided_large_workspace_bytes(n: int, num_systems: int, elem_stride: int, sy
 
 
 def _pad_n(n: int) -> int:
-    p = 2
-    while p < n:
-        p <<= 1
-    return p
+    return 1 << max(1, (int(n) - 1).bit_length())
 
 
 def max_switch_level(dtype, algo, n: int) -> int:
@@ -234,27 +249,37 @@ def solve_batched(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, stream=None
     """
     if x is None:
         x = torch.empty_strided(d.shape, d.stride(), dtype=d.dtype, device=d.device)
-    _check_tensors([a, b, c, d, x], "cuda", same_strides=True)
-    S, n = d.shape
-    ss, es = d.stride()
-    if stream is None:
-        stream = torch.cuda.current_stream(d.device)
+    # cheap common-case validation (the per-call host cost matters for small
+    # batches); anything unusual goes through the full check for its message
+    shape, strides, dt, dev = d.shape, d.stride(), d.dtype, d.device
+    if (len(shape) != 2 or not d.is_cuda or dt not in DTYPES
+            or any(t.shape != shape or t.dtype != dt or t.stride() != strides or t.device != dev
+                   for t in (a, b, c, x))):
+        _check_tensors([a, b, c, d, x], "cuda", same_strides=True)
+    S, n = shape
+    ss, es = strides
     contiguous = es == 1 and (ss == n or S <= 1)
-    if (_pad_n(n) > max_n(d.dtype, algo) and contiguous
-            and _pad_n(n) <= max_n_large(d.dtype, algo)):
-        return solve_batched_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
-                                   stream=stream)
-    if not contiguous:
+    if contiguous:
+        pn = _pad_n(n)
+        if pn > max_n(dt, algo) and pn <= max_n_large(dt, algo):
+            return solve_batched_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
+                                       stream=stream)
+    else:
         # pitched rows / interleaved columns: the workspace entry point (column
         # or row passes where the on-chip strided kernels would be slow or
         # too small; none needed otherwise)
         return solve_batched_strided_large(a, b, c, d, x, algo=algo, switch_level=switch_level,
                                            stream=stream)
-    with torch.cuda.device(d.device):
-        st = solve_batched_raw(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
-                               x.data_ptr(), n, S, d.dtype, algo, switch_level,
-                               stream.cuda_stream)
-    check(st)
+    L = _lib if _lib is not None else load()
+    if dev.index != _current_device():
+        with torch.cuda.device(dev):
+            return solve_batched(a, b, c, d, x=x, algo=algo, switch_level=switch_level, stream=stream)
+    raw = _current_raw_stream(dev.index) if stream is None else stream.cuda_stream
+    st = L.tridiag_solve_batched(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                 x.data_ptr(), n, S, DTYPES[dt], _algo_code(algo),
+                                 int(switch_level), raw)
+    if st != 0:
+        check(st)
     return x
 
 
