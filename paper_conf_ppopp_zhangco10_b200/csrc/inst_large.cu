@@ -42,15 +42,21 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
       auto kern = tdg::tdg_large_heads_kernel<T, R, K>;
       const int64_t units = S * (C - 1);
       const int grid = (int)std::min<int64_t>((units + 127) / 128, 148LL * 16);
-      { const cudaError_t le_ = launch_k(kern, dim3(grid), dim3(128), 0, st, a, b, c, d, hbuf, n, n_real, ss, S, (int)CH, vec ? 1 : 0, c_pad); if (le_ != cudaSuccess) return le_; }
+      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(128), 0, st, a, b, c, d, hbuf, n, n_real, ss, S, (int)CH, vec ? 1 :
+          0, c_pad);
+      if (lerr != cudaSuccess) return lerr;
     } else if (which == 1) {
       auto kern = tdg::tdg_large_reduce_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
-      { const cudaError_t le_ = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, o1, o2, o3, hbuf, n, n_real, ss, S, vec ? 1 : 0, c_pad); if (le_ != cudaSuccess) return le_; }
+      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, o1, o2, o3, hbuf, n, n_real, ss, S,
+          vec ? 1 : 0, c_pad);
+      if (lerr != cudaSuccess) return lerr;
     } else {
       auto kern = tdg::tdg_large_expand_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
-      { const cudaError_t le_ = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, hbuf, n, n_real, ss, S, vec ? 1 : 0, c_pad); if (le_ != cudaSuccess) return le_; }
+      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, hbuf, n, n_real, ss, S, vec ? 1
+          : 0, c_pad);
+      if (lerr != cudaSuccess) return lerr;
     }
     return cudaGetLastError();
   };

@@ -33,8 +33,9 @@ cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x
   const int64_t tiles = (S + G - 1) / G;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)device_sms(dev) * occ));
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(threads), smem, st, a, b, c, d, x, (int)n, (long long)S, k, lp,
-                                              (int)n_real, c_pad, (long long)L.es); if (le_ != cudaSuccess) return le_; }
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(threads), smem, st, a, b, c, d, x, (int)n, (long long)S, k,
+      lp, (int)n_real, c_pad, (long long)L.es);
+  if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   return cudaGetLastError();
 }
@@ -71,9 +72,9 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(threads), smem, st, a, b, c, d, x, (int)n, (long long)S, k, log2P,
-                                           vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es,
-                                           (long long)L.ss, stamps); if (le_ != cudaSuccess) return le_; }
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(threads), smem, st, a, b, c, d, x, (int)n, (long long)S, k,
+      log2P, vec ? 1 : 0, pf, (int)n_real, c_pad, (long long)L.es, (long long)L.ss, stamps);
+  if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   return cudaGetLastError();
 }
@@ -158,7 +159,9 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
     }
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode()); if (le_ != cudaSuccess) return le_; }
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long
+      long)S, k, dbuf, tma_pf_mode());
+  if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   *used = true;
   return cudaGetLastError();
@@ -261,8 +264,9 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   const int pm = prefetch_mode();
   const int pf = vec && (pm == 1 || pm == 2) ? 1 : 0;
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
-  { const cudaError_t le_ = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem, st, a, b, c, d, x, (int)n, (long long)S, k, vec ? 1 : 0, pf,
-                                             (int)nr, c_pad, (long long)L.es, (long long)L.ss); if (le_ != cudaSuccess) return le_; }
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem, st, a, b, c, d, x, (int)n, (long long)S, k,
+      vec ? 1 : 0, pf, (int)nr, c_pad, (long long)L.es, (long long)L.ss);
+  if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   return cudaGetLastError();
 }
