@@ -45,6 +45,8 @@ PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 int pdl_mode();
 // L2 prefetch of the unit after the one a TMA kernel is copying (TRIDIAG_TMA_PF).
 int tma_pf_mode();
+// TMA CTA kernel for ragged contiguous rows (TRIDIAG_RAG_TMA, default 1).
+int rag_tma_mode();
 // Double-buffered CTA-kernel regions (TRIDIAG_CTA_DBUF, default 1).
 int cta_dbuf_mode();
 // 2-CTA cluster kernel for 16-warp systems (opt-in TRIDIAG_CTA_CLUSTER=1).

@@ -114,25 +114,58 @@ bool make_row_map(CUtensorMap* m, const void* base, int64_t rows, int R, int box
   return r == CUDA_SUCCESS;
 }
 
+// Ragged contiguous rows (system stride n_real): 3-D map {R, ceil(n_real/R), S}
+// with strides {R T, n_real T} (tdg_cta_tma_kernel<..., RAG = true>).
+template <typename T>
+bool make_rag_map(CUtensorMap* m, const void* base, int64_t n_real, int64_t S, int R, int box_rows) {
+  auto fn = encode_fn();
+  if (!fn) return false;
+  if ((reinterpret_cast<uintptr_t>(base) & 15) != 0 || ((uint64_t)n_real * sizeof(T)) % 16 != 0) return false;
+  const int64_t rows = (n_real + R - 1) / R;
+  if (S >= (int64_t(1) << 31) || rows >= (int64_t(1) << 31)) return false;
+  const cuuint64_t dims[3] = {(cuuint64_t)R, (cuuint64_t)rows, (cuuint64_t)S};
+  const cuuint64_t strides[2] = {(cuuint64_t)R * sizeof(T), (cuuint64_t)n_real * sizeof(T)};
+  const cuuint32_t box[3] = {(cuuint32_t)R, (cuuint32_t)box_rows, 1};
+  const cuuint32_t estr[3] = {1, 1, 1};
+  const CUresult r = fn(m, sizeof(T) == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64,
+                        3, const_cast<void*>(base), dims, strides, box, estr,
+                        CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_64B,
+                        CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS;
+}
+
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                           int64_t S, int k, cudaStream_t st, bool* used) {
+                           int64_t S, int k, cudaStream_t st, bool* used, int64_t nr = -1) {
   *used = false;
   const int P = 32 * W;
+  const bool rag = nr >= 0 && nr != n;
+  if (nr < 0) nr = n;
   const int64_t rows = S * P;
   if (rows >= (int64_t(1) << 31)) return cudaSuccess;
   CUtensorMap mA, mB, mC, mD;
   const int box = P > 256 ? 256 : P;
-  if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
-      !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box))
+  if (rag) {
+    if ((reinterpret_cast<uintptr_t>(x) & 15) != 0 || !make_rag_map<T>(&mA, a, nr, S, R, box) ||
+        !make_rag_map<T>(&mB, b, nr, S, R, box) || !make_rag_map<T>(&mC, c, nr, S, R, box) ||
+        !make_rag_map<T>(&mD, d, nr, S, R, box))
+      return cudaSuccess;
+  } else if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
+             !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box)) {
     return cudaSuccess;
+  }
   const size_t smem = tdg::cta_tma_smem_bytes<T>(R, W, INNER, k);
   int dev = 0;
   cudaGetDevice(&dev);
   constexpr int LR = ilog2c(R);
   auto kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, -1>;
+  if (rag) {
+    // register path only (k >= log2 R; RD: k > log2 R)
+    if (k < LR || (INNER == tdg::kRD && k == LR)) return cudaSuccess;
+    kern = tdg::tdg_cta_tma_kernel<T, R, W, INNER, -1, true>;
+  }
   // RD with k <= log2 R (one survivor per lane at k = log2 R): blocked CTA scan
-  if (k < LR || (INNER == tdg::kRD && k == LR)) {
+  if (!rag && (k < LR || (INNER == tdg::kRD && k == LR))) {
     if constexpr (INNER != tdg::kRD) {
       return cudaSuccess;
     } else {
@@ -159,8 +192,7 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
     }
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long
-      long)S, k, dbuf, tma_pf_mode());
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode(), (int)nr);
   if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   *used = true;
@@ -236,6 +268,13 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
       tma_mode()) {
     bool used = false;
     const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used);
+    if (used || e != cudaSuccess) return e;
+  }
+  // ragged contiguous rows with 16-byte aligned systems: the TMA kernel with
+  // 3-D maps (rows past the system zero-filled, padding in registers)
+  if (nr != n && L.es == 1 && L.ss == nr && tma_mode() && rag_tma_mode()) {
+    bool used = false;
+    const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used, nr);
     if (used || e != cudaSuccess) return e;
   }
   const bool staged = (nr != n || !vec) && L.es == 1;

@@ -50,6 +50,15 @@ __device__ __forceinline__ void tma_load_2d(void* dst, const CUtensorMap* map, i
       : "memory");
 }
 
+__device__ __forceinline__ void tma_load_3d(void* dst, const CUtensorMap* map, int c0, int c1, int c2,
+                                            uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3, %4}], [%5];" ::"r"(
+          smem_u32(dst)),
+      "l"(reinterpret_cast<uint64_t>(map)), "r"(c0), "r"(c1), "r"(c2), "r"(smem_u32(bar))
+      : "memory");
+}
+
 // L2 prefetch of a TMA box (no shared memory, no completion): issued for the
 // unit after the one being copied, it keeps two units per CTA in flight to
 // HBM while the stage holds only one.
@@ -86,11 +95,17 @@ __host__ __device__ constexpr uint32_t tma_stage_bytes(int R, int W) {
 
 // KB = -1: k >= log2 R (register path); KB >= 0: RD inner with k = KB
 // (cta_blocked_rd).
-template <typename T, int R, int W, int INNER, int KB>
+// RAG = true: ragged contiguous rows (n_real < n, system stride n_real, n_real
+// T a multiple of 16 B).  The tensor maps are 3-D {R, ceil(n_real / R), S}
+// with strides {R T, n_real T}: a system's 64-byte rows, the last one running
+// into the next system, rows past the system zero-filled by TMA; equations
+// i >= n_real become the padding equations of reading R26 in registers and
+// only the real ones are stored.
+template <typename T, int R, int W, int INNER, int KB, bool RAG = false>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
-                   T* x, int n, long long S, int k, int dbuf, int pf) {
+                   T* x, int n, long long S, int k, int dbuf, int pf, int n_real) {
   pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
@@ -112,9 +127,12 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     for (int q = 0; q < 4; ++q)
 #pragma unroll
       for (int bx = 0; bx < NBOX; ++bx)
-        tma_load_2d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0,
-                    (int)(sys * P + bx * ROWS), bar);
-    if (pf && sys + gridDim.x < S) {
+        if constexpr (RAG)
+          tma_load_3d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0, bx * ROWS, (int)sys, bar);
+        else
+          tma_load_2d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0,
+                      (int)(sys * P + bx * ROWS), bar);
+    if (!RAG && pf && sys + gridDim.x < S) {
 #pragma unroll
       for (int q = 0; q < 4; ++q)
 #pragma unroll
@@ -144,6 +162,17 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     read_row<T, R>(stage + 1 * ARR_BYTES + ls * 64, sw, rb);
     read_row<T, R>(stage + 2 * ARR_BYTES + ls * 64, sw, rc);
     read_row<T, R>(stage + 3 * ARR_BYTES + ls * 64, sw, rd);
+    if constexpr (RAG) {
+      const int i0 = ls * R;
+      if (i0 + R >= n_real) {  // this lane holds c_{n_real-1} or padding rows
+        const T c_pad = INNER == kRD ? T(1) : T(0);
+#pragma unroll
+        for (int t = 0; t < R; ++t) {
+          if (i0 + t >= n_real) { ra[t] = T(0); rb[t] = T(1); rc[t] = c_pad; rd[t] = T(0); }
+          if (i0 + t == n_real - 1) rc[t] = c_pad;
+        }
+      }
+    }
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     const long long next = sys + gridDim.x;
@@ -159,7 +188,26 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
       xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
     }
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
-    store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
+    if constexpr (RAG) {
+      T* p = x + (size_t)sys * (size_t)n_real + (size_t)ls * R;
+      if (ls * R + R <= n_real) {
+        // 16-byte aligned (n_real T and R T are multiples of 16 B)
+#pragma unroll
+        for (int q = 0; q < R * (int)sizeof(T) / 16; ++q) {
+          constexpr int E = 16 / (int)sizeof(T);
+          if constexpr (sizeof(T) == 4)
+            *reinterpret_cast<float4*>(p + q * E) = make_float4(rd[q * E], rd[q * E + 1], rd[q * E + 2], rd[q * E + 3]);
+          else
+            *reinterpret_cast<double2*>(p + q * E) = make_double2(rd[q * E], rd[q * E + 1]);
+        }
+      } else {
+#pragma unroll
+        for (int t = 0; t < R; ++t)
+          if (ls * R + t < n_real) p[t] = rd[t];
+      }
+    } else {
+      store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
+    }
     if (dbuf == 0) __syncthreads();  // heads / survivor regions are reused by the next system
   }
 }

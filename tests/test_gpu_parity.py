@@ -561,3 +561,31 @@ def test_full_size_other_configs_sampled(name, dtype, S, n, algo, fam, res_tol, 
     idx = torch.randperm(S, generator=torch.Generator().manual_seed(1))[:samples].cuda()
     e = err_vs_oracle(a[idx], b[idx], c[idx], d[idx], x[idx])
     assert e.max() <= TOL[dtype], (name, e.max())
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_ragged_cta_tma_bitwise_equal_staged(dtype, monkeypatch):
+    """Ragged contiguous rows beyond one warp (n_pad > 32 R) with 16-byte
+    aligned systems take the TMA CTA kernel with 3-D maps (rows past the
+    system zero-filled, padding equations in registers): bitwise equal to the
+    staged general path (same operations on the same padded system), within
+    the gates, and the neighbouring systems' elements are never written."""
+    R = 16 if dtype == torch.float32 else 8
+    step = 4 if dtype == torch.float32 else 2
+    for n in (33 * R - step, 1000, 64 * R + step, 3000, 4000, 128 * R * 2 - 4 * step):
+        if n % step or n > td.max_n(dtype, "cr"):
+            continue
+        for algo, m, fam in (("cr", 0, "dd"), ("cr_pcr", 0, "dd"), ("cr_pcr", 2, "dd"), ("cr_rd", 32, "rdw")):
+            S = 37
+            a, b, c, d = gen(fam, S, n, dtype, seed=n + m)
+            guard = torch.full((S * n + 64,), 7.0, dtype=dtype, device="cuda")
+            x1 = guard[:S * n].view(S, n)
+            monkeypatch.setenv("TRIDIAG_RAG_TMA", "1")
+            td.solve_batched(a, b, c, d, x=x1, algo=algo, switch_level=m)
+            torch.cuda.synchronize()
+            monkeypatch.setenv("TRIDIAG_RAG_TMA", "0")
+            x0 = gpu_solve(a, b, c, d, algo, m)
+            assert torch.equal(x1, x0), (n, algo, m, (x1 - x0).abs().max().item())
+            assert bool((guard[S * n:] == 7.0).all()), (n, algo, m)
+            assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, algo, m)
+    monkeypatch.delenv("TRIDIAG_RAG_TMA")

@@ -34,6 +34,8 @@ CASES = [
     (torch.float64, 2048, 40, "cr", 0, "column"),        # column passes fp64, two levels
     (torch.float32, 2048, 64, "cr_pcr", 0, "column_fused"),  # single-kernel column sweep
     (torch.float64, 1000, 40, "cr_rd", 0, "column_fused"),   # same, fp64, ragged n, RD inner
+    (torch.float32, 1000, 9, "cr_pcr", 0, "contig"),     # ragged rows: TMA CTA kernel, 3-D maps
+    (torch.float64, 3000, 5, "cr_rd", 0, "contig"),      # same, fp64, RD inner
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
