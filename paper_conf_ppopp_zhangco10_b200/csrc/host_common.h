@@ -45,7 +45,8 @@ PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 int pdl_mode();
 // L2 prefetch of the unit after the one a TMA kernel is copying (TRIDIAG_TMA_PF).
 int tma_pf_mode();
-// TMA CTA kernel for ragged contiguous rows (TRIDIAG_RAG_TMA, default 1).
+// Vector paths for ragged contiguous rows: the TMA CTA kernel with 3-D maps
+// and the warp kernel's per-lane 16-byte accesses (TRIDIAG_RAG_TMA, default 1).
 int rag_tma_mode();
 // Double-buffered CTA-kernel regions (TRIDIAG_CTA_DBUF, default 1).
 int cta_dbuf_mode();

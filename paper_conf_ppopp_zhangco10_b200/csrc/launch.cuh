@@ -57,12 +57,21 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // registers); every other instantiation asks for two CTAs per SM
   // (TRIDIAG_BLOCKED_MINB=1 at run time selects the unconstrained build for
   // the blocked inner instead, for A/B measurements).
-  auto kern = (KB < 0 && vec) ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
+  // ragged contiguous rows with 16-byte aligned systems: per-lane vector
+  // accesses, no staging (register path)
+  const bool rag = KB < 0 && !vec && n_real != n && L.es == 1 && L.ss == n_real &&
+                   (R * sizeof(T)) % 16 == 0 && ((uint64_t)n_real * sizeof(T)) % 16 == 0 &&
+                   ((reinterpret_cast<uintptr_t>(a) | reinterpret_cast<uintptr_t>(b) |
+                     reinterpret_cast<uintptr_t>(c) | reinterpret_cast<uintptr_t>(d) |
+                     reinterpret_cast<uintptr_t>(x)) & 15) == 0 &&
+                   rag_tma_mode();
+  auto kern = rag ? tdg::tdg_warp_kernel<T, R, INNER, KB, false, true>
+            : (KB < 0 && vec) ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
             : (KB < 0)        ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>
             : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
                                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
                   : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
-  const size_t tiles = vec ? 0 : (((size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15));
+  const size_t tiles = (vec || rag) ? 0 : (((size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15));
   const size_t smem = tiles + (size_t)wpb * tdg::pcr_scratch_bytes<T, R, INNER, KB>();
   const int occ = occupancy(dev, kern, threads, smem);
   if (occ <= 0) return cudaErrorInvalidConfiguration;

@@ -148,7 +148,48 @@ __device__ __forceinline__ void staged_store(T* x, long long s0, long long S, lo
 // loads only).  GEN = true: the general path -- scalar loads, element / system
 // strides, padded (ragged) n -- compiled separately so the fast path carries
 // none of its registers.
-template <typename T, int R, int INNER, int KB, bool GEN>
+// RAG = true (with GEN = false): ragged contiguous rows (system stride
+// n_real, n_real T a multiple of 16 B, 16-byte aligned pointers): each lane
+// moves its R equations with 16-byte vector accesses when they are all real,
+// element by element (padding equations of reading R26 past n_real) at the
+// end of a system -- no shared-memory staging.
+template <typename T, int R, bool NC>
+__device__ __forceinline__ void load_block16(const T* p, T (&v)[R]) {
+  constexpr int E = 16 / (int)sizeof(T);
+  if constexpr (R % E != 0) {  // (not launched: the host requires 16-byte lane blocks)
+#pragma unroll
+    for (int t = 0; t < R; ++t) v[t] = p[t];
+    return;
+  }
+#pragma unroll
+  for (int q = 0; q < R / E; ++q) {
+    if constexpr (sizeof(T) == 4) {
+      const float4 t = NC ? __ldg(reinterpret_cast<const float4*>(p) + q) : reinterpret_cast<const float4*>(p)[q];
+      v[q * 4] = t.x; v[q * 4 + 1] = t.y; v[q * 4 + 2] = t.z; v[q * 4 + 3] = t.w;
+    } else {
+      const double2 t = NC ? __ldg(reinterpret_cast<const double2*>(p) + q) : reinterpret_cast<const double2*>(p)[q];
+      v[q * 2] = t.x; v[q * 2 + 1] = t.y;
+    }
+  }
+}
+template <typename T, int R>
+__device__ __forceinline__ void store_block16(T* p, const T (&v)[R]) {
+  constexpr int E = 16 / (int)sizeof(T);
+  if constexpr (R % E != 0) {  // (not launched: the host requires 16-byte lane blocks)
+#pragma unroll
+    for (int t = 0; t < R; ++t) p[t] = v[t];
+    return;
+  }
+#pragma unroll
+  for (int q = 0; q < R / E; ++q) {
+    if constexpr (sizeof(T) == 4)
+      reinterpret_cast<float4*>(p)[q] = make_float4(v[q * 4], v[q * 4 + 1], v[q * 4 + 2], v[q * 4 + 3]);
+    else
+      reinterpret_cast<double2*>(p)[q] = make_double2(v[q * 2], v[q * 2 + 1]);
+  }
+}
+
+template <typename T, int R, int INNER, int KB, bool GEN, bool RAG = false>
 __device__ __forceinline__ void warp_kernel_body(
     const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c, const T* d, T* x,
     int n, long long S, int k, int log2P, int vec, int pf, int n_real, T c_pad, long long es,
@@ -186,7 +227,29 @@ __device__ __forceinline__ void warp_kernel_body(
     const size_t sbase = (size_t)sys * (size_t)ss;
     const size_t off = sbase + (size_t)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
-    if constexpr (!GEN) {
+    if constexpr (RAG) {
+      const int i0 = ls * R;
+      if (valid && i0 + R <= n_real) {
+        load_block16<T, R, true>(a + off, ra);
+        load_block16<T, R, true>(b + off, rb);
+        load_block16<T, R, true>(c + off, rc);
+        load_block16<T, R, false>(d + off, rd);
+      } else {
+#pragma unroll
+        for (int t = 0; t < R; ++t) {
+          const bool in = valid && i0 + t < n_real;
+          ra[t] = in ? a[off + t] : T(0);
+          rb[t] = in ? b[off + t] : T(1);
+          rc[t] = in ? c[off + t] : c_pad;
+          rd[t] = in ? d[off + t] : T(0);
+        }
+      }
+      if (i0 + R >= n_real) {
+#pragma unroll
+        for (int t = 0; t < R; ++t)
+          if (i0 + t == n_real - 1) rc[t] = c_pad;  // c_{n_real-1} (R26)
+      }
+    } else if constexpr (!GEN) {
       if (valid) {
         load_block<T, R, true>(a + off, ra, vec);
         load_block<T, R, true>(b + off, rb, vec);
@@ -208,7 +271,18 @@ __device__ __forceinline__ void warp_kernel_body(
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp, pcr_scr);
-    if constexpr (!GEN) {
+    if constexpr (RAG) {
+      const int i0 = ls * R;
+      if (valid) {
+        if (i0 + R <= n_real) {
+          store_block16<T, R>(x + off, rd);
+        } else {
+#pragma unroll
+          for (int t = 0; t < R; ++t)
+            if (i0 + t < n_real) x[off + t] = rd[t];
+        }
+      }
+    } else if constexpr (!GEN) {
       if (valid) store_block<T, R>(x + off, rd, vec);
     } else {
       staged_store<T, R>(x, s0, S, ss, n, n_real, log2P + ilog2c(R), lane, rd, warp_tile<T, R>(warp));
@@ -219,14 +293,14 @@ __device__ __forceinline__ void warp_kernel_body(
 
 // KB < 0 (the register path of the tuned hybrids and CR): ptxas picks ~127
 // registers for 256 threads, two CTAs (16 warps) per SM.
-template <typename T, int R, int INNER, int KB, bool GEN>
+template <typename T, int R, int INNER, int KB, bool GEN, bool RAG = false>
 __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                 int n_real, T c_pad, long long es, long long ss, long long* stamps) {
   pdl_entry();
-  warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
-                                         es, ss, stamps);
+  warp_kernel_body<T, R, INNER, KB, GEN, RAG>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
+                                              es, ss, stamps);
 }
 
 // KB >= 0 (register-blocked inner: PCR, RD, large m) is latency bound with

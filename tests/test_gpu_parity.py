@@ -589,3 +589,29 @@ def test_ragged_cta_tma_bitwise_equal_staged(dtype, monkeypatch):
             assert bool((guard[S * n:] == 7.0).all()), (n, algo, m)
             assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, algo, m)
     monkeypatch.delenv("TRIDIAG_RAG_TMA")
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_ragged_warp_vector_bitwise_equal_staged(dtype, monkeypatch):
+    """Ragged contiguous rows within one warp (n_pad <= 32 R) with 16-byte
+    aligned systems: per-lane 16-byte accesses instead of the staged path --
+    bitwise the same x (same padded system), within the gates, corners
+    poisoned, guard elements after the batch untouched; small and large
+    batches (both lane plans)."""
+    step = 4 if dtype == torch.float32 else 2
+    for n in (12, 36, 100, 244, 500, 508) if dtype == torch.float32 else (10, 30, 100, 250):
+        for S in (5, 3001):
+            for algo, m, fam in (("cr", 0, "dd"), ("cr_pcr", 0, "dd"), ("cr_rd", 0, "rdw")):
+                a, b, c, d = gen(fam, S, n, dtype, seed=n + S, poison_corners=True)
+                guard = torch.full((S * n + 64,), 7.0, dtype=dtype, device="cuda")
+                x1 = guard[:S * n].view(S, n)
+                monkeypatch.setenv("TRIDIAG_RAG_TMA", "1")
+                td.solve_batched(a, b, c, d, x=x1, algo=algo, switch_level=m)
+                torch.cuda.synchronize()
+                monkeypatch.setenv("TRIDIAG_RAG_TMA", "0")
+                x0 = gpu_solve(a, b, c, d, algo, m)
+                assert torch.equal(x1, x0), (n, S, algo)
+                assert bool((guard[S * n:] == 7.0).all()), (n, S, algo)
+                if algo != "cr_rd" or n <= 64:
+                    assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, S, algo)
+    monkeypatch.delenv("TRIDIAG_RAG_TMA")

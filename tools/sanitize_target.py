@@ -36,6 +36,8 @@ CASES = [
     (torch.float64, 1000, 40, "cr_rd", 0, "column_fused"),   # same, fp64, ragged n, RD inner
     (torch.float32, 1000, 9, "cr_pcr", 0, "contig"),     # ragged rows: TMA CTA kernel, 3-D maps
     (torch.float64, 3000, 5, "cr_rd", 0, "contig"),      # same, fp64, RD inner
+    (torch.float32, 500, 37, "cr_pcr", 0, "contig"),     # ragged rows: warp kernel, 16-byte lanes
+    (torch.float64, 100, 41, "cr", 0, "contig"),         # same, fp64, 4 lanes per system
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
