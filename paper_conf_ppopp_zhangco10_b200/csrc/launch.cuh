@@ -59,8 +59,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // the blocked inner instead, for A/B measurements).
   // ragged contiguous rows with 16-byte aligned systems: per-lane vector
   // accesses, no staging (register path)
-  const bool rag = KB < 0 && !vec && n_real != n && L.es == 1 && L.ss == n_real &&
-                   (R * sizeof(T)) % 16 == 0 && ((uint64_t)n_real * sizeof(T)) % 16 == 0 &&
+  const bool rag = KB < 0 && !vec && L.es == 1 && (L.ss >= n_real || S <= 1) &&
+                   (R * sizeof(T)) % 16 == 0 && ((uint64_t)L.ss * sizeof(T)) % 16 == 0 &&
                    ((reinterpret_cast<uintptr_t>(a) | reinterpret_cast<uintptr_t>(b) |
                      reinterpret_cast<uintptr_t>(c) | reinterpret_cast<uintptr_t>(d) |
                      reinterpret_cast<uintptr_t>(x)) & 15) == 0 &&
@@ -123,17 +123,18 @@ bool make_row_map(CUtensorMap* m, const void* base, int64_t rows, int R, int box
   return r == CUDA_SUCCESS;
 }
 
-// Ragged contiguous rows (system stride n_real): 3-D map {R, ceil(n_real/R), S}
-// with strides {R T, n_real T} (tdg_cta_tma_kernel<..., RAG = true>).
+// Ragged and / or pitched rows (system stride ss >= n_real, ss T a multiple of
+// 16 B): 3-D map {R, ceil(n_real/R), S} with strides {R T, ss T}
+// (tdg_cta_tma_kernel<..., RAG = true>).
 template <typename T>
-bool make_rag_map(CUtensorMap* m, const void* base, int64_t n_real, int64_t S, int R, int box_rows) {
+bool make_rag_map(CUtensorMap* m, const void* base, int64_t n_real, int64_t ss, int64_t S, int R, int box_rows) {
   auto fn = encode_fn();
   if (!fn) return false;
-  if ((reinterpret_cast<uintptr_t>(base) & 15) != 0 || ((uint64_t)n_real * sizeof(T)) % 16 != 0) return false;
+  if ((reinterpret_cast<uintptr_t>(base) & 15) != 0 || ((uint64_t)ss * sizeof(T)) % 16 != 0) return false;
   const int64_t rows = (n_real + R - 1) / R;
   if (S >= (int64_t(1) << 31) || rows >= (int64_t(1) << 31)) return false;
   const cuuint64_t dims[3] = {(cuuint64_t)R, (cuuint64_t)rows, (cuuint64_t)S};
-  const cuuint64_t strides[2] = {(cuuint64_t)R * sizeof(T), (cuuint64_t)n_real * sizeof(T)};
+  const cuuint64_t strides[2] = {(cuuint64_t)R * sizeof(T), (cuuint64_t)ss * sizeof(T)};
   const cuuint32_t box[3] = {(cuuint32_t)R, (cuuint32_t)box_rows, 1};
   const cuuint32_t estr[3] = {1, 1, 1};
   const CUresult r = fn(m, sizeof(T) == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64,
@@ -145,19 +146,21 @@ bool make_rag_map(CUtensorMap* m, const void* base, int64_t n_real, int64_t S, i
 
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                           int64_t S, int k, cudaStream_t st, bool* used, int64_t nr = -1) {
+                           int64_t S, int k, cudaStream_t st, bool* used, int64_t nr = -1,
+                           int64_t ss = -1) {
   *used = false;
   const int P = 32 * W;
-  const bool rag = nr >= 0 && nr != n;
   if (nr < 0) nr = n;
+  if (ss < 0) ss = n;
+  const bool rag = nr != n || ss != n;
   const int64_t rows = S * P;
   if (rows >= (int64_t(1) << 31)) return cudaSuccess;
   CUtensorMap mA, mB, mC, mD;
   const int box = P > 256 ? 256 : P;
   if (rag) {
-    if ((reinterpret_cast<uintptr_t>(x) & 15) != 0 || !make_rag_map<T>(&mA, a, nr, S, R, box) ||
-        !make_rag_map<T>(&mB, b, nr, S, R, box) || !make_rag_map<T>(&mC, c, nr, S, R, box) ||
-        !make_rag_map<T>(&mD, d, nr, S, R, box))
+    if ((reinterpret_cast<uintptr_t>(x) & 15) != 0 || !make_rag_map<T>(&mA, a, nr, ss, S, R, box) ||
+        !make_rag_map<T>(&mB, b, nr, ss, S, R, box) || !make_rag_map<T>(&mC, c, nr, ss, S, R, box) ||
+        !make_rag_map<T>(&mD, d, nr, ss, S, R, box))
       return cudaSuccess;
   } else if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
              !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box)) {
@@ -201,7 +204,8 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
     }
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
-  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode(), (int)nr);
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode(), (int)nr,
+                                    (long long)ss);
   if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   *used = true;
@@ -281,9 +285,10 @@ cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int
   }
   // ragged contiguous rows with 16-byte aligned systems: the TMA kernel with
   // 3-D maps (rows past the system zero-filled, padding in registers)
-  if (nr != n && L.es == 1 && L.ss == nr && tma_mode() && rag_tma_mode()) {
+  if ((nr != n || L.ss != n) && L.es == 1 && (L.ss >= nr || S <= 1) && tma_mode() && rag_tma_mode()) {
     bool used = false;
-    const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used, nr);
+    const int64_t ss = S <= 1 ? std::max<int64_t>(nr, (L.ss * (int64_t)sizeof(T) % 16) ? ((nr + 3) & ~3LL) : L.ss) : L.ss;
+    const cudaError_t e = launch_cta_tma<T, R, W, INNER>(a, b, c, d, x, n, S, k, st, &used, nr, ss);
     if (used || e != cudaSuccess) return e;
   }
   const bool staged = (nr != n || !vec) && L.es == 1;

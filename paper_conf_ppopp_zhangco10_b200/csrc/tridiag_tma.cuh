@@ -95,17 +95,17 @@ __host__ __device__ constexpr uint32_t tma_stage_bytes(int R, int W) {
 
 // KB = -1: k >= log2 R (register path); KB >= 0: RD inner with k = KB
 // (cta_blocked_rd).
-// RAG = true: ragged contiguous rows (n_real < n, system stride n_real, n_real
-// T a multiple of 16 B).  The tensor maps are 3-D {R, ceil(n_real / R), S}
-// with strides {R T, n_real T}: a system's 64-byte rows, the last one running
-// into the next system, rows past the system zero-filled by TMA; equations
-// i >= n_real become the padding equations of reading R26 in registers and
-// only the real ones are stored.
+// RAG = true: ragged and / or pitched rows (n_real <= n, system stride ss >=
+// n_real, ss T a multiple of 16 B).  The tensor maps are 3-D
+// {R, ceil(n_real / R), S} with strides {R T, ss T}: a system's 64-byte rows,
+// the last one possibly running past the system, rows past it zero-filled by
+// TMA; equations i >= n_real become the padding equations of reading R26 in
+// registers and only the real ones are stored.
 template <typename T, int R, int W, int INNER, int KB, bool RAG = false>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
-                   T* x, int n, long long S, int k, int dbuf, int pf, int n_real) {
+                   T* x, int n, long long S, int k, int dbuf, int pf, int n_real, long long ss) {
   pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
@@ -189,7 +189,7 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     }
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
     if constexpr (RAG) {
-      T* p = x + (size_t)sys * (size_t)n_real + (size_t)ls * R;
+      T* p = x + (size_t)sys * (size_t)ss + (size_t)ls * R;
       if (ls * R + R <= n_real) {
         // 16-byte aligned (n_real T and R T are multiples of 16 B)
 #pragma unroll

@@ -615,3 +615,27 @@ def test_ragged_warp_vector_bitwise_equal_staged(dtype, monkeypatch):
                 if algo != "cr_rd" or n <= 64:
                     assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, S, algo)
     monkeypatch.delenv("TRIDIAG_RAG_TMA")
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_pitched_rows_vector_paths(dtype, monkeypatch):
+    """Pitched rows (system stride > n, a multiple of 16 bytes) take the same
+    vector paths (warp kernel 16-byte lanes; TMA CTA kernel with 3-D maps):
+    bitwise equal to the contiguous solve of the same systems, the gap
+    between rows untouched."""
+    for n in (100, 500, 512, 1000, 1024, 4096):
+        if n > td.max_n(dtype, "cr"):
+            continue
+        pitch = n + (16 if dtype == torch.float32 else 8) + (4 - n % 4) % 4
+        S = 45
+        rows = gen("dd", S, n, dtype, seed=n + 5)
+        bufs = [torch.full((S, pitch), 3.0, dtype=dtype, device="cuda") for _ in range(5)]
+        views = []
+        for bf, t in zip(bufs, list(rows) + [rows[0]]):
+            bf[:, :n] = t
+            views.append(bf[:, :n])
+        ref = td.solve_batched(*rows, algo="cr_pcr")
+        x = td.solve_batched(*views[:4], x=views[4], algo="cr_pcr")
+        torch.cuda.synchronize()
+        assert torch.equal(x, ref), n
+        assert bool((bufs[4][:, n:] == 3.0).all()), n

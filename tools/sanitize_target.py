@@ -38,6 +38,8 @@ CASES = [
     (torch.float64, 3000, 5, "cr_rd", 0, "contig"),      # same, fp64, RD inner
     (torch.float32, 500, 37, "cr_pcr", 0, "contig"),     # ragged rows: warp kernel, 16-byte lanes
     (torch.float64, 100, 41, "cr", 0, "contig"),         # same, fp64, 4 lanes per system
+    (torch.float32, 1000, 9, "cr_pcr", 0, "pitched"),    # pitched ragged rows: TMA 3-D maps
+    (torch.float32, 500, 37, "cr", 0, "pitched"),        # pitched ragged rows: warp 16-byte lanes
 ]
 
 only = int(sys.argv[1]) if len(sys.argv) > 1 else None
@@ -50,6 +52,12 @@ for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
     os.environ["TRIDIAG_COL_FUSED"] = "1" if layout == "column_fused" else "0"
     if layout in ("column", "column_fused"):
         views = [t.t().contiguous().t() for t in (a, b, c, d)]
+    elif layout == "pitched":
+        views = []
+        for t in (a, b, c, d):
+            bf = torch.zeros((S, n + 12), dtype=dt, device="cuda")
+            bf[:, :n] = t
+            views.append(bf[:, :n])
     else:
         views = [a, b, c, d]
     x = td.solve_batched(*views, algo=algo, switch_level=m)
