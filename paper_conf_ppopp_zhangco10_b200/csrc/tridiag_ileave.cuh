@@ -79,6 +79,29 @@ __device__ __forceinline__ void ilv_issue(const T* a, const T* b, const T* c, co
   unsigned so = (unsigned)__cvta_generic_to_shared(tile) + (unsigned)(r0 * G + g) * sizeof(T);
   const unsigned TB = (unsigned)TE * sizeof(T);
   const bool all_rows = row0 + P * R <= n_real - 1;  // no padding row, no c_{n_real-1} here
+  if (sys_ok && all_rows) {
+    // the common case (every row real, the system exists): branch-free copies
+#pragma unroll 4
+    for (int j = 0; j < R; ++j, pa += step, pb += step, pc += step, pd += step) {
+      const int r = r0 + P * j;
+      const unsigned sj = so + (unsigned)(P * j * G + (r >> 4)) * sizeof(T);
+      if constexpr (sizeof(T) == 4) {
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj), "l"(pa) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + TB), "l"(pb) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + 2 * TB), "l"(pc) : "memory");
+        if (COPY_D)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(sj + 3 * TB), "l"(pd) : "memory");
+      } else {
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj), "l"(pa) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + TB), "l"(pb) : "memory");
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + 2 * TB), "l"(pc) : "memory");
+        if (COPY_D)
+          asm volatile("cp.async.ca.shared.global [%0], [%1], 8;" ::"r"(sj + 3 * TB), "l"(pd) : "memory");
+      }
+    }
+    cp_async_commit();
+    return;
+  }
 #pragma unroll 4
   for (int j = 0; j < R; ++j, pa += step, pb += step, pc += step, pd += step) {
     // (r0 + P j) >> 4 == (P j) >> 4 + (r0 >> 4) for P | 16 or 16 | P
@@ -123,6 +146,14 @@ __device__ __forceinline__ void ilv_writeback(T* x, const T* tX, long long t0, l
   const long long step = (long long)P * es;
   const T* srcp = tX + r0 * G + g;
   const bool all_rows = row0 + P * R <= n_real;
+  if (all_rows) {
+#pragma unroll 4
+    for (int j = 0; j < R; ++j, dst += step) {
+      const int r = r0 + P * j;
+      *dst = srcp[P * j * G + (r >> 4)];
+    }
+    return;
+  }
 #pragma unroll 4
   for (int j = 0; j < R; ++j, dst += step) {
     const int r = r0 + P * j;
