@@ -100,8 +100,13 @@ enum {
  *
  * Pointers must be device memory of the current device.  Alignment: the
  * vector path needs every pointer aligned to the per-thread tile
- * (min(32, R*sizeof(T)) bytes); otherwise a scalar-load path runs (same
- * results).  Results are deterministic: bitwise identical across runs and
+ * (min(32, R*sizeof(T)) bytes); ragged n with n*sizeof(T) a multiple of 16
+ * and 16-byte aligned pointers takes 16-byte / TMA vector paths; otherwise a
+ * staged scalar-load path runs (bitwise the same results in every case).
+ * Launches carry the programmatic-dependent-launch attribute: a kernel's
+ * thread blocks may be scheduled while the previous work on the stream
+ * drains, but every kernel waits for it (griddepcontrol.wait) before its
+ * first memory access, so stream order is unchanged.  Results are deterministic: bitwise identical across runs and
  * across any partitioning of the batch.  Numeric failure (a zero pivot; RD
  * overflow outside its stable regime) is not an error code: it
  * shows up as non-finite x (no pivoting).
@@ -123,9 +128,11 @@ int tridiag_solve_batched(const void* a, const void* b, const void* c, const voi
  * es >= num_systems is the ADI column sweep of a row-major grid ("the most
  * common application", ADI): e.g. the columns of an
  * NY x NX grid are NX systems of n = NY with elem_stride = NX, sys_stride = 1.
- * Interleaved layouts are staged through shared memory in tiles of 8
- * consecutive systems (coalesced 32-byte rows); other non-contiguous layouts
- * use scalar loads.  x must use the same strides; x == d is allowed.
+ * Interleaved layouts are staged through shared memory in tiles of 8-32
+ * consecutive systems (coalesced row segments); pitched rows whose pitch is
+ * a multiple of 16 bytes take the same vector paths as contiguous rows;
+ * other non-contiguous layouts use scalar loads.  x must use the same
+ * strides; x == d is allowed.
  * Errors as tridiag_solve_batched plus TRIDIAG_ERR_STRIDE.
  */
 int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, const void* d,
