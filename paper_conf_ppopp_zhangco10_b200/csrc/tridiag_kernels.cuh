@@ -22,6 +22,11 @@
 #ifndef TDG_BLOCKED_MINB
 #define TDG_BLOCKED_MINB 2
 #endif
+// CTAs per SM the LU-form RD kernel asks for (its three scans want ~185
+// registers: 1 CTA of 8 warps, or 2 with spills)
+#ifndef TDG_STONE_MINB
+#define TDG_STONE_MINB 2
+#endif
 
 namespace tdg {
 
@@ -308,7 +313,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 // registers; the few spills land in the otherwise unused L1) doubles the
 // warps that hide the shuffle / MUFU latency.
 template <typename T, int R, int INNER, int KB, bool GEN>
-__global__ void __launch_bounds__(256, (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : 1)
+__global__ void __launch_bounds__(256, (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
