@@ -73,7 +73,7 @@ int env_int(const char* name, int dflt) {
   const char* v = getenv(name);
   return (v && *v) ? atoi(v) : dflt;
 }
-int g_force_R = -1, g_prefetch = -1;
+int g_force_R = -1;
 int force_R() { if (g_force_R < 0) g_force_R = env_int("TRIDIAG_WARP_R", 0); return g_force_R; }
 
 }  // namespace

@@ -116,7 +116,7 @@ tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
-  extern __shared__ __align__(16) unsigned char smem_raw[];
+  extern __shared__ __align__(1024) unsigned char smem_raw[];
   T* pages = reinterpret_cast<T*>(smem_raw);  // [2][W][HE]
   T* carry = pages + 2 * W * HE;              // [2][HE]
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;

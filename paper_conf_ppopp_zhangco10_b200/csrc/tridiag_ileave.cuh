@@ -174,7 +174,7 @@ tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __r
                   const T* d, T* x, int n, long long S, int k, int log2P, int n_real, T c_pad,
                   long long es) {
   pdl_entry();
-  extern __shared__ __align__(16) unsigned char smem_raw[];
+  extern __shared__ __align__(1024) unsigned char smem_raw[];
   T* tile = reinterpret_cast<T*>(smem_raw);
   const IlvGeom<LP> Gm(log2P);
   const int G = Gm.G(), P = Gm.P();

@@ -85,7 +85,7 @@ template <typename T, int R>
 __host__ __device__ constexpr int warp_tile_elems() { return 32 * R + R + 1; }
 template <typename T, int R>
 __device__ __forceinline__ T* warp_tile(int warp) {
-  extern __shared__ __align__(16) unsigned char smem_raw[];
+  extern __shared__ __align__(1024) unsigned char smem_raw[];
   return reinterpret_cast<T*>(smem_raw) + (size_t)warp * 4 * warp_tile_elems<T, R>();
 }
 __device__ __forceinline__ int wt_off(int q) { return q + (q >> 5); }
@@ -164,16 +164,16 @@ __device__ __forceinline__ void load_block16(const T* p, T (&v)[R]) {
   if constexpr (R % E != 0) {  // (not launched: the host requires 16-byte lane blocks)
 #pragma unroll
     for (int t = 0; t < R; ++t) v[t] = p[t];
-    return;
-  }
+  } else {
 #pragma unroll
-  for (int q = 0; q < R / E; ++q) {
-    if constexpr (sizeof(T) == 4) {
-      const float4 t = NC ? __ldg(reinterpret_cast<const float4*>(p) + q) : reinterpret_cast<const float4*>(p)[q];
-      v[q * 4] = t.x; v[q * 4 + 1] = t.y; v[q * 4 + 2] = t.z; v[q * 4 + 3] = t.w;
-    } else {
-      const double2 t = NC ? __ldg(reinterpret_cast<const double2*>(p) + q) : reinterpret_cast<const double2*>(p)[q];
-      v[q * 2] = t.x; v[q * 2 + 1] = t.y;
+    for (int q = 0; q < R / E; ++q) {
+      if constexpr (sizeof(T) == 4) {
+        const float4 t = NC ? __ldg(reinterpret_cast<const float4*>(p) + q) : reinterpret_cast<const float4*>(p)[q];
+        v[q * 4] = t.x; v[q * 4 + 1] = t.y; v[q * 4 + 2] = t.z; v[q * 4 + 3] = t.w;
+      } else {
+        const double2 t = NC ? __ldg(reinterpret_cast<const double2*>(p) + q) : reinterpret_cast<const double2*>(p)[q];
+        v[q * 2] = t.x; v[q * 2 + 1] = t.y;
+      }
     }
   }
 }
@@ -183,14 +183,14 @@ __device__ __forceinline__ void store_block16(T* p, const T (&v)[R]) {
   if constexpr (R % E != 0) {  // (not launched: the host requires 16-byte lane blocks)
 #pragma unroll
     for (int t = 0; t < R; ++t) p[t] = v[t];
-    return;
-  }
+  } else {
 #pragma unroll
-  for (int q = 0; q < R / E; ++q) {
-    if constexpr (sizeof(T) == 4)
-      reinterpret_cast<float4*>(p)[q] = make_float4(v[q * 4], v[q * 4 + 1], v[q * 4 + 2], v[q * 4 + 3]);
-    else
-      reinterpret_cast<double2*>(p)[q] = make_double2(v[q * 2], v[q * 2 + 1]);
+    for (int q = 0; q < R / E; ++q) {
+      if constexpr (sizeof(T) == 4)
+        reinterpret_cast<float4*>(p)[q] = make_float4(v[q * 4], v[q * 4 + 1], v[q * 4 + 2], v[q * 4 + 3]);
+      else
+        reinterpret_cast<double2*>(p)[q] = make_double2(v[q * 2], v[q * 2 + 1]);
+    }
   }
 }
 
@@ -210,7 +210,7 @@ __device__ __forceinline__ void warp_kernel_body(
   // per-warp scratch of the cyclic PCR relayout, after the GEN warp tiles
   T* pcr_scr = nullptr;
   if constexpr (pcr_scratch_bytes<T, R, INNER, KB>() > 0) {
-    extern __shared__ __align__(16) unsigned char smem_raw[];
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
     const size_t off = GEN ? (((size_t)wpb * 4 * warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15)) : 0;
     pcr_scr = reinterpret_cast<T*>(smem_raw + off + (size_t)warp * pcr_scratch_bytes<T, R, INNER, KB>());
   }
@@ -608,7 +608,7 @@ tdg_cta_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __rest
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;
-  extern __shared__ __align__(16) unsigned char smem_raw[];
+  extern __shared__ __align__(1024) unsigned char smem_raw[];
   T* smem = reinterpret_cast<T*>(smem_raw);
   T* heads = smem;                        // W * LRH * 4
   T* work = smem + W * LRH * 4;
