@@ -43,6 +43,8 @@ PFN_cuTensorMapEncodeTiled_v12000 encode_fn();
 
 // Programmatic dependent launch (TRIDIAG_PDL, default 1): see pdl_entry().
 int pdl_mode();
+// Smaller warp-kernel CTAs for batches below 8 warps per SM (TRIDIAG_SMALL_CTA).
+int small_cta_mode();
 // L2 prefetch of the unit after the one a TMA kernel is copying (TRIDIAG_TMA_PF).
 int tma_pf_mode();
 // Vector paths for ragged contiguous rows: the TMA CTA kernel with 3-D maps

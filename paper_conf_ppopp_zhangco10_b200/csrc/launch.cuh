@@ -47,10 +47,18 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int P = (int)(n / R);
   const int log2P = ilog2c(P);
   const int G = 32 / P;
-  const int wpb = 8;
-  const int threads = wpb * 32;
   int dev = 0;
   cudaGetDevice(&dev);
+  // 8 warps per CTA; a batch too small to give every SM 8 warps is spread
+  // over all SMs in smaller CTAs instead (fewer warps per scheduler: the
+  // latency-bound regime of the paper-sized batches, e.g. 512 x 512)
+  int wpb = 8;
+  {
+    const int64_t warps_needed = (S + G - 1) / G;
+    const int64_t sms = device_sms(dev);
+    while (wpb > 1 && warps_needed < sms * wpb && small_cta_mode()) wpb >>= 1;
+  }
+  const int threads = wpb * 32;
   // vec: the contiguous power-of-two vector path; otherwise the general
   // (scalar / strided / padded) instantiation
   // The tuned register path (KB < 0, vector) lets ptxas choose (~127

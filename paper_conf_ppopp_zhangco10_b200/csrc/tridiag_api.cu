@@ -93,6 +93,7 @@ int cta_dbuf_mode() {
 }
 int rag_tma_mode() { return env_int("TRIDIAG_RAG_TMA", 1); }  // read per call (A/B)
 int tma_pf_mode() { return env_int("TRIDIAG_TMA_PF", 0); }  // opt-in (measured: -1 to -8 points on rows); read per call
+int small_cta_mode() { return env_int("TRIDIAG_SMALL_CTA", 1); }  // read per call (A/B)
 int pdl_mode() {
   static int v = -1;
   if (v < 0) v = env_int("TRIDIAG_PDL", 1);
