@@ -411,7 +411,10 @@ def main():
                 ("c4_f32_1048576x256", "f32", 256, 1 << 20, "rows", "cr_pcr", "dd"),
                 ("c5_f32_16384x8192", "f32", 8192, 16384, "rows", "cr_pcr", "dd"),
                 ("large_f32_64x1048576", "f32", 1 << 20, 64, "rows", "cr_pcr", "dd"),
-                ("large_f64_32x1048576", "f64", 1 << 20, 32, "rows", "cr_pcr", "dd")):
+                ("large_f64_32x1048576", "f64", 1 << 20, 32, "rows", "cr_pcr", "dd"),
+                # ragged n (not a power of two; padded in-kernel, NEXT f2)
+                ("ragged_f32_67108x1000", "f32", 1000, 67108, "rows", "cr_pcr", "dd"),
+                ("ragged_f32_134217x500", "f32", 500, 134217, "rows", "cr_pcr", "dd")):
             dtt = torch.float32 if dts == "f32" else torch.float64
             TT = 4 if dts == "f32" else 8
             sets = []
