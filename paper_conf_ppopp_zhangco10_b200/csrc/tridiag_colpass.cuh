@@ -236,7 +236,10 @@ __host__ __device__ constexpr uint32_t col_stage_bytes() { return 4u * 32u * W *
 
 template <typename T, int R, int W>
 __host__ __device__ constexpr size_t col_reduce_tma_smem() {
-  return col_stage_bytes<T, R, W>() + 16 + col_reduce_smem<T, R, W>();
+  // one page of W warps' heads (the unit-start barrier that frees the stage
+  // also orders the next unit's head stores after this unit's reads) plus
+  // the two carry pages
+  return col_stage_bytes<T, R, W>() + 16 + (size_t)(W + 2) * col_heads_elems<T, R>() * sizeof(T);
 }
 
 template <typename T, int R, int W>
@@ -284,8 +287,8 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
   extern __shared__ __align__(1024) unsigned char smem_raw[];
   unsigned char* stage = smem_raw;
   uint64_t* bar = reinterpret_cast<uint64_t*>(smem_raw + 4 * ARR);
-  T* pages = reinterpret_cast<T*>(smem_raw + 4 * ARR + 16);  // [2][W][HE]
-  T* carry = pages + 2 * W * HE;                              // [2][HE]
+  T* pages = reinterpret_cast<T*>(smem_raw + 4 * ARR + 16);  // [W][HE]
+  T* carry = pages + W * HE;                                  // [2][HE]
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   const long long C = n / CH;
   const long long U = ((S + 31) >> 5) * C;
@@ -314,7 +317,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     const long long g = u / C, ch = u - g * C;
     const long long s = g * 32 + lane;
     const bool sok = s < S;
-    T* pg = pages + (j & 1) * W * HE;
+    T* pg = pages;
     T* cin = carry + ((j + 1) & 1) * HE;
     if (j == 0 && ch + 1 < C && w == 0) {
       T ha[R], hb[R], hc[R], hd[R];
