@@ -48,7 +48,8 @@ struct Stamp {
 
 // KB < 0: k >= LR (all in-lane levels; m <= P, lane-level inner solve).
 // KB >= 0: k == KB < LR (m = P * (R >> KB) > P, register-blocked inner solve).
-template <typename T, int R, int INNER, int KB>
+// PCR_CYC: pcr_scratch is the warp's cyclic-relayout scratch (blocked PCR).
+template <typename T, int R, int INNER, int KB, bool PCR_CYC = false>
 __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&d)[R], int k,
                                            int ls, int P, Stamp st = Stamp(),
                                            T* pcr_scratch = nullptr) {
@@ -68,7 +69,7 @@ __device__ __forceinline__ void warp_solve(T (&a)[R], T (&b)[R], T (&c)[R], T (&
   } else {
     // m = P * (R >> KB) > P: the intermediate system stays block-distributed
     // in registers (no copy; the paper copies it to 5 extra arrays).
-    if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P, pcr_scratch);
+    if constexpr (INNER == kPCR) blocked_pcr<T, R, (KB < 0 ? 0 : KB), PCR_CYC>(a, b, c, d, ls, P, pcr_scratch);
     else blocked_rd<T, R, (KB < 0 ? 0 : KB)>(a, b, c, d, ls, P);
   }
   st.mark(3);
@@ -275,7 +276,7 @@ __device__ __forceinline__ void warp_kernel_body(
     // a_0 and c_{n-1} are not matrix entries: never read.
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
-    warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, stp, pcr_scr);
+    warp_solve<T, R, INNER, KB, (pcr_scratch_bytes<T, R, INNER, KB>() > 0)>(ra, rb, rc, rd, k, ls, P, stp, pcr_scr);
     if constexpr (RAG) {
       const int i0 = ls * R;
       if (valid) {
