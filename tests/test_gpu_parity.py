@@ -347,6 +347,38 @@ def test_corner_poisoning_is_ignored(dtype):
             assert torch.equal(gpu_solve(*p1, algo), gpu_solve(*p2, algo)), (algo, n)
 
 
+@pytest.mark.parametrize("n,algo,m", [(64, "pcr", 0), (512, "pcr", 0), (512, "cr_pcr", 256),
+                                       (512, "cr_pcr", 32), (4096, "cr_pcr", 0)])
+def test_broken_system_does_not_touch_its_neighbours(n, algo, m):
+    """A zero pivot b_0 = 0 in one system (no pivoting) sends
+    the reciprocal batch of its warp down the rcp.rn slow path; every other
+    system must come out bitwise identical to the run without it (the slow
+    path is rcp.rn itself, and absent neighbours never cross systems)."""
+    a, b, c, d = gen("dd", 70, n, torch.float32)
+    x0 = gpu_solve(a, b, c, d, algo, m)
+    bad = [0, 5, 33, 69]
+    b2 = b.clone()
+    b2[bad, 0] = 0.0
+    x1 = gpu_solve(a, b2, c, d, algo, m)
+    keep = [i for i in range(70) if i not in bad]
+    assert torch.equal(x0[keep], x1[keep])
+
+
+@pytest.mark.parametrize("algo,m", [("pcr", 0), ("cr_pcr", 256), ("cr_pcr", 0), ("cr", 0)])
+def test_huge_coefficients_take_the_rcp_slow_path(algo, m):
+    """Every coefficient scaled by 2^125: pivots reach [2^126, 2^128), outside
+    the fast reciprocal's range, so the batch is recomputed with rcp.rn (whose
+    results are subnormal there).  The solution is scale-invariant
+    (A x = d is homogeneous in (a, b, c, d)); gate G1 against the oracle."""
+    a, b, c, d = gen("dd", 263, 512, torch.float32)
+    s = 2.0 ** 125
+    a, b, c, d = a * s, b * s, c * s, d * s  # exact: powers of two, no overflow (|b| < 4)
+    assert torch.isfinite(b).all() and b.abs().max() >= 2.0 ** 126
+    x = gpu_solve(a, b, c, d, algo, m)
+    assert torch.isfinite(x).all()
+    assert err_vs_oracle(a, b, c, d, x) < TOL[torch.float32]
+
+
 def test_in_place_x_equals_d():
     for dtype in (torch.float32, torch.float64):
         for n in [64, 512, 4096]:
