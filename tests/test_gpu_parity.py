@@ -365,18 +365,26 @@ def test_broken_system_does_not_touch_its_neighbours(n, algo, m):
 
 
 @pytest.mark.parametrize("algo,m", [("pcr", 0), ("cr_pcr", 256), ("cr_pcr", 0), ("cr", 0)])
-def test_huge_coefficients_take_the_rcp_slow_path(algo, m):
-    """Every coefficient scaled by 2^125: pivots reach [2^126, 2^128), outside
-    the fast reciprocal's range, so the batch is recomputed with rcp.rn (whose
-    results are subnormal there).  The solution is scale-invariant
-    (A x = d is homogeneous in (a, b, c, d)); gate G1 against the oracle."""
+def test_huge_rows_take_the_rcp_slow_path(algo, m):
+    """Strongly dominant systems (|a|, |c| < 1/16, 1 <= |b| < 2) whose
+    equations i < n/2 are scaled by 2^126 (row scaling leaves x unchanged):
+    those pivots lie in [2^126, 2^127), outside the fast reciprocal's range,
+    so their reciprocal batches are recomputed with rcp.rn.  Every row keeps
+    its own scale through CR/PCR, the pivots grow by < 2x (dominance), and
+    each final 2x2 pair has one row of each half, so nothing overflows.
+    (At |b| up to 4 * 2^125, plain DD, pivot growth overflows fp32: the
+    method has no scaling.)  Gate G1 against the oracle."""
     a, b, c, d = gen("dd", 263, 512, torch.float32)
-    s = 2.0 ** 125
-    a, b, c, d = a * s, b * s, c * s, d * s  # exact: powers of two, no overflow (|b| < 4)
+    a, c = a / 16, c / 16
+    b = torch.sign(b) * (1 + (b.abs() - 1) / 3)  # |b| in [1, 2)
+    sc = torch.ones(512, device="cuda", dtype=torch.float32)
+    sc[:256] = 2.0 ** 126
+    a, b, c, d = a * sc, b * sc, c * sc, d * sc  # exact: powers of two
     assert torch.isfinite(b).all() and b.abs().max() >= 2.0 ** 126
     x = gpu_solve(a, b, c, d, algo, m)
     assert torch.isfinite(x).all()
-    assert err_vs_oracle(a, b, c, d, x) < TOL[torch.float32]
+    e = err_vs_oracle(a, b, c, d, x)
+    assert e.max() <= TOL[torch.float32], e.max()
 
 
 def test_in_place_x_equals_d():
