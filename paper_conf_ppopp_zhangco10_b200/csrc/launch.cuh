@@ -52,7 +52,7 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // 8 warps per CTA; a batch too small to give every SM 8 warps is spread
   // over all SMs in smaller CTAs instead (fewer warps per scheduler: the
   // latency-bound regime of the paper-sized batches, e.g. 512 x 512)
-  int wpb = 8;
+  int wpb = (vec && blocked_minb() != 1 && tdg::pcr_small_cta<T, R, INNER, KB, false>()) ? 4 : 8;
   {
     const int64_t warps_needed = (S + G - 1) / G;
     const int64_t sms = device_sms(dev);
