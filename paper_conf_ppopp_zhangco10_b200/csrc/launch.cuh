@@ -52,7 +52,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // 8 warps per CTA; a batch too small to give every SM 8 warps is spread
   // over all SMs in smaller CTAs instead (fewer warps per scheduler: the
   // latency-bound regime of the paper-sized batches, e.g. 512 x 512)
-  int wpb = (vec && blocked_minb() != 1 && tdg::pcr_small_cta<T, R, INNER, KB, false>()) ? 4 : 8;
+  const bool small = vec && blocked_minb() != 1 && P >= 16 && tdg::pcr_small_cta<T, R, INNER, KB, false>();
+  int wpb = small ? 4 : 8;
   {
     const int64_t warps_needed = (S + G - 1) / G;
     const int64_t sms = device_sms(dev);
@@ -73,10 +74,17 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
                      reinterpret_cast<uintptr_t>(c) | reinterpret_cast<uintptr_t>(d) |
                      reinterpret_cast<uintptr_t>(x)) & 15) == 0 &&
                    rag_tma_mode();
+  auto small_kern = [] {
+    if constexpr (tdg::pcr_small_cta<T, R, INNER, KB, false>())
+      return tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true>;
+    else
+      return tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>;
+  }();
   auto kern = rag ? tdg::tdg_warp_kernel<T, R, INNER, KB, false, true>
             : (KB < 0 && vec) ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
             : (KB < 0)        ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>
             : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
+                     : small             ? small_kern
                                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
                   : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
   const size_t tiles = (vec || rag) ? 0 : (((size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15));

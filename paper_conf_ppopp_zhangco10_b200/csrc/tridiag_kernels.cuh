@@ -313,16 +313,16 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 // one 8-warp CTA per SM at ~170 registers; asking for two CTAs (<= 128
 // registers; the few spills land in the otherwise unused L1) doubles the
 // warps that hide the shuffle / MUFU latency.
-// PCR alone at n = 512 fp32 (k = 0, vector path): 4-warp CTAs, 3 per SM,
-// 170 registers (12 warps per SM without the 2-CTA spills).
+// SMALL: PCR alone in fp32 (k = 0, vector path, P >= 16 lanes per system):
+// 4-warp CTAs, 3 per SM, 170 registers (12 warps per SM, fewer spills than
+// at the 2-CTA cap); n = 64 / 128 (P < 16) are faster with the default.
 template <typename T, int R, int INNER, int KB, bool GEN>
 __host__ __device__ constexpr bool pcr_small_cta() {
   return INNER == kPCR && KB == 0 && !GEN && sizeof(T) == 4 && R == 16;
 }
-template <typename T, int R, int INNER, int KB, bool GEN>
-__global__ void __launch_bounds__(pcr_small_cta<T, R, INNER, KB, GEN>() ? 128 : 256,
-                                  pcr_small_cta<T, R, INNER, KB, GEN>() ? 3
-                                  : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
+template <typename T, int R, int INNER, int KB, bool GEN, bool SMALL = false>
+__global__ void __launch_bounds__(SMALL ? 128 : 256,
+                                  SMALL ? 3 : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
