@@ -318,7 +318,7 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 // at the 2-CTA cap); n = 64 / 128 (P < 16) are faster with the default.
 template <typename T, int R, int INNER, int KB, bool GEN>
 __host__ __device__ constexpr bool pcr_small_cta() {
-  return INNER == kPCR && KB == 0 && !GEN && sizeof(T) == 4 && R == 16;
+  return INNER == kPCR && (KB == 0 || KB == 1) && !GEN && sizeof(T) == 4 && R == 16;
 }
 template <typename T, int R, int INNER, int KB, bool GEN, bool SMALL = false>
 __global__ void __launch_bounds__(SMALL ? 128 : 256,
