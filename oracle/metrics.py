@@ -26,13 +26,17 @@ def tridiag_matvec(a, b, c, x):
 
 
 def normwise_error(x, xhat):
-    """Per-system max_i |x_i - xhat_i| / max_i |xhat_i| (inf if x has a non-finite)."""
+    """Per-system max_i |x_i - xhat_i| / max_i |xhat_i| over the last axis.
+
+    inf if x has a non-finite entry; 0 when x equals xhat exactly (0/0, the
+    d = 0 system, reading R18). Pinned by tests/test_oracle.py
+    ``test_normwise_error_*`` (hand-computed exact values)."""
     x = np.asarray(x, dtype=np.float64)
     xhat = np.asarray(xhat, dtype=np.float64)
     num = np.max(np.abs(x - xhat), axis=-1)
     den = np.max(np.abs(xhat), axis=-1)
     with np.errstate(invalid="ignore", divide="ignore"):
-        e = num / den
+        e = np.where(num == 0.0, 0.0, num / den)
     bad = ~np.all(np.isfinite(x), axis=-1)
     e = np.where(bad, np.inf, e)
     return e

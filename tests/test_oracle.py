@@ -402,3 +402,75 @@ def test_rd_stone_dense_small_and_no_overflow():
     x32, _ = oracle.rd_stone(a, b, c, d, dtype=np.float32)
     assert np.all(np.isfinite(x32))
     assert oracle.normwise_error(x32, oracle.thomas(a, b, c, d)).max() <= 1e-5
+
+
+# ----------------------------------------------------------------------------- the error metric (R18)
+# Every parity gate is decided by normwise_error, so it is pinned on values
+# computed by hand (powers of two, so every expected value is exact in fp64):
+# a dropped abs, a reduction over the wrong axis, a division by max|x|
+# instead of max|x^|, a sum instead of a max, fp32 evaluation or a lost
+# non-finite check each fails one of these.
+def test_normwise_error_single_perturbation_is_delta_over_max_abs_xhat():
+    xhat = np.array([1.0, -4.0, 2.0])
+    x = xhat.copy()
+    x[2] += 2.0 ** -10
+    assert oracle.normwise_error(x, xhat) == 2.0 ** -10 / 4.0
+
+
+def test_normwise_error_counts_through_abs():
+    # numerator: a sign flip (x - x^ negative) must count
+    assert oracle.normwise_error(np.array([-1.0, 2.0]), np.array([1.0, 2.0])) == 1.0
+    # denominator: the largest |x^_i| is a negative entry
+    xhat = np.array([-8.0, 1.0])
+    x = np.array([-8.0, 1.0 + 2.0 ** -3])
+    assert oracle.normwise_error(x, xhat) == 2.0 ** -3 / 8.0
+
+
+def test_normwise_error_divides_by_the_reference_not_the_result():
+    assert oracle.normwise_error(np.array([8.0, 0.0]), np.array([4.0, 0.0])) == 1.0
+
+
+def test_normwise_error_is_a_max_not_a_sum():
+    xhat = np.ones(4)
+    x = xhat + 2.0 ** -5
+    assert oracle.normwise_error(x, xhat) == 2.0 ** -5
+
+
+def test_normwise_error_reduces_per_system():
+    xhat = np.array([[1.0, 1.0, 1.0], [100.0, 100.0, 100.0], [-2.0, 0.5, 0.25]])
+    x = xhat.copy()
+    x[0, 2] += 2.0 ** -4
+    x[2, 1] -= 2.0 ** -6
+    e = oracle.normwise_error(x, xhat)
+    assert e.shape == (3,)
+    assert list(e) == [2.0 ** -4, 0.0, 2.0 ** -6 / 2.0]
+
+
+def test_normwise_error_evaluates_in_fp64():
+    xhat = np.array([3.0], np.float32)
+    x = np.nextafter(xhat, np.float32(4.0))        # 3 + 2^-22
+    assert oracle.normwise_error(x, xhat)[()] == 2.0 ** -22 / 3.0
+
+
+def test_normwise_error_non_finite_is_inf():
+    xhat = np.array([[1.0, 2.0], [1.0, 2.0], [1.0, 2.0]])
+    x = np.array([[1.0, np.nan], [np.inf, 2.0], [1.0, 2.0]])
+    assert list(oracle.normwise_error(x, xhat)) == [np.inf, np.inf, 0.0]
+
+
+def test_normwise_error_exact_zero_system():
+    # d = 0 gives x = x^ = 0: no error (0/0 read as 0, R18); any x != 0 is inf
+    assert oracle.normwise_error(np.zeros(3), np.zeros(3)) == 0.0
+    assert oracle.normwise_error(np.array([0.0, 1e-300, 0.0]), np.zeros(3)) == np.inf
+
+
+def test_normwise_error_on_a_real_solve_matches_its_definition_by_hand():
+    # a solve perturbed in one component of one system: exactly that system moves
+    a, b, c, d = gen("dd", 5, 64, seed=77)
+    xhat = oracle.thomas(a, b, c, d)
+    x = xhat.copy()
+    x[3, 17] += 1e-6
+    e = oracle.normwise_error(x, xhat)
+    assert list(e[[0, 1, 2, 4]]) == [0.0] * 4
+    by_hand = abs((xhat[3, 17] + 1e-6) - xhat[3, 17]) / max(abs(v) for v in xhat[3])
+    assert e[3] == by_hand
