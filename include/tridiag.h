@@ -271,6 +271,14 @@ int64_t tridiag_max_switch_level(int dtype, int algo, int64_t n);
  * invalid arguments. */
 int tridiag_auto_switch_level(int64_t n, int dtype, int algo);
 
+/* Re-read the TRIDIAG_* tuning knobs from the environment (diagnostic: A/B
+ * measurements and the bitwise path-equality tests).  Normally the knobs are
+ * read once, on the library's first call, and never change afterwards; calling
+ * this while another thread is solving is allowed (each knob is an atomic) but
+ * that solve may see either value.  No effect on results except which of
+ * several bitwise-equal kernels runs. */
+void tridiag_reload_knobs(void);
+
 /* TRIDIAG_ABI_VERSION of the loaded library. */
 int tridiag_abi_version(void);
 

@@ -52,8 +52,8 @@ int tma_pf_mode();
 int rag_tma_mode();
 // Double-buffered CTA-kernel regions (TRIDIAG_CTA_DBUF, default 1).
 int cta_dbuf_mode();
-// 2-CTA cluster kernel for 16-warp systems (opt-in TRIDIAG_CTA_CLUSTER=1).
-int cta_cluster_mode();
+// TMA-fed column passes (TRIDIAG_COL_TMA, default 1).
+int col_tma_mode();
 
 // Launch with the programmatic-stream-serialization attribute (when enabled):
 // the kernel's CTAs may be scheduled while the previous grid on the stream
@@ -122,17 +122,5 @@ template <typename T>
 cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, T* o0, T* o1,
                      T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t es, int64_t S,
                      int64_t es2, int kin, T c_pad, cudaStream_t st);
-
-// Single-pass column sweep (tridiag_colfused.cuh, inst_colfused.cu): shape
-// eligibility, workspace bytes, and the launch (false = not applicable for
-// these pointers / this device; *err = launch status otherwise).
-template <typename T>
-bool col_fused_eligible(int64_t n, int inner, int64_t m);
-template <typename T>
-size_t col_fused_ws_bytes(int64_t n, int64_t S);
-template <typename T>
-bool col_fused(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n, int64_t n_real,
-               int64_t es, int64_t S, int inner, int64_t m, T c_pad, void* ws, cudaStream_t st,
-               cudaError_t* err);
 
 }  // namespace tdg_host

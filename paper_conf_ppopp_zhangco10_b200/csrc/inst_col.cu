@@ -44,14 +44,6 @@ bool make_col_map(CUtensorMap* m, const void* base, int64_t S, int64_t rows, int
   return r == CUDA_SUCCESS;
 }
 
-int col_tma_mode() {
-  static int v = -1;
-  if (v < 0) {
-    const char* e = getenv("TRIDIAG_COL_TMA");
-    v = (e && *e) ? atoi(e) : 1;
-  }
-  return v;
-}
 }  // namespace
 
 template <typename T>

@@ -5,7 +5,6 @@
 #include "host_common.h"
 #include "tridiag_ileave.cuh"
 #include "tridiag_tma.cuh"
-#include "tridiag_cta2.cuh"
 
 namespace tdg_host {
 
@@ -228,71 +227,9 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
   return cudaGetLastError();
 }
 
-// A system of 2 x 32 W lanes on a 2-CTA cluster (tridiag_cta2.cuh): the
-// register path only (k >= log2 R, and for RD k > log2 R), at most 32
-// survivors after the lane-level levels.  *used = false: not applicable.
-template <typename T, int R, int W, int INNER>
-cudaError_t launch_cta2_tma(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                            int64_t S, int k, cudaStream_t st, bool* used) {
-  *used = false;
-  constexpr int LR = ilog2c(R);
-  constexpr int CL = 2;
-  const int P = 32 * W;
-  if (!cta_cluster_mode() || n != (int64_t)CL * P * R) return cudaSuccess;
-  if (k < LR || (INNER == tdg::kRD && k == LR)) return cudaSuccess;
-  const int kl = std::min(k - LR, 5);
-  if (CL * W * (32 >> kl) > 32) return cudaSuccess;
-  const int64_t rows = S * CL * P;
-  if (rows >= (int64_t(1) << 31)) return cudaSuccess;
-  CUtensorMap mA, mB, mC, mD;
-  const int box = P > 256 ? 256 : P;
-  if (!make_row_map<T>(&mA, a, rows, R, box) || !make_row_map<T>(&mB, b, rows, R, box) ||
-      !make_row_map<T>(&mC, c, rows, R, box) || !make_row_map<T>(&mD, d, rows, R, box))
-    return cudaSuccess;
-  auto kern = tdg::tdg_cta2_tma_kernel<T, R, W, INNER>;
-  const size_t smem = tdg::cta2_smem_bytes<T, R, W>();
-  int dev = 0;
-  cudaGetDevice(&dev);
-  if (smem > 48 * 1024) cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  cudaLaunchConfig_t cfg = {};
-  cfg.blockDim = dim3(W * 32);
-  cfg.dynamicSmemBytes = smem;
-  cfg.stream = st;
-  cudaLaunchAttribute at[2];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = CL;
-  at[0].val.clusterDim.y = 1;
-  at[0].val.clusterDim.z = 1;
-  at[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-  at[1].val.programmaticStreamSerializationAllowed = 1;
-  cfg.attrs = at;
-  cfg.numAttrs = 1;
-  cfg.gridDim = dim3(CL);
-  int maxc = 0;
-  if (cudaOccupancyMaxActiveClusters(&maxc, kern, &cfg) != cudaSuccess || maxc <= 0) {
-    cudaGetLastError();
-    return cudaSuccess;
-  }
-  const int64_t ncl = std::max<int64_t>(1, std::min<int64_t>(S, maxc));
-  cfg.gridDim = dim3((unsigned)(ncl * CL));
-  cfg.numAttrs = pdl_mode() ? 2 : 1;
-  const cudaError_t e = cudaLaunchKernelEx(&cfg, kern, mA, mB, mC, mD, x, (int)n, (long long)S, k);
-  if (e != cudaSuccess) return e;
-  g_last_launches = 1;
-  *used = true;
-  return cudaSuccess;
-}
-
 template <typename T, int R, int W, int INNER>
 cudaError_t launch_cta(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
                        int64_t S, int k, bool vec, cudaStream_t st, int64_t nr, Layout L) {
-  if constexpr (W == 16) {
-    if (vec && nr == n && L.es == 1 && L.ss == n && tma_mode()) {
-      bool used = false;
-      const cudaError_t e = launch_cta2_tma<T, R, 8, INNER>(a, b, c, d, x, n, S, k, st, &used);
-      if (used || e != cudaSuccess) return e;
-    }
-  }
   if (vec && nr == n && L.es == 1 && L.ss == n && (k >= ilog2c(R) || INNER == tdg::kRD) &&
       tma_mode()) {
     bool used = false;

@@ -4,6 +4,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <atomic>
 #include <cstdint>
 #include <cstdlib>
 #include <cstring>
@@ -66,48 +67,63 @@ int auto_m(int64_t n, int dtype, int algo) {
 }
 
 
-// Tuning knobs (environment, read once): TRIDIAG_WARP_R forces R of the warp
-// kernel when n/R <= 32; TRIDIAG_PREFETCH=0/1 disables/enables the L2 bulk
-// prefetch of the next system.  Defaults come from the sweeps in profiles/.
+// Tuning knobs (environment).  Read ONCE, on the first call of the library
+// (std::call_once), into atomics: the launch plan never changes mid-process
+// and no solve pays a getenv.  tridiag_reload_knobs() re-reads them (A/B
+// measurements and the bitwise path-equality tests only).  Defaults are the
+// tuned paths (profiles/r01_tune_plan.md):
+//   TRIDIAG_WARP_R       force R of the warp kernel (0 = plan)
+//   TRIDIAG_PREFETCH     L2 bulk prefetch of the next system (2 = auto)
+//   TRIDIAG_CTA_DBUF     double-buffered CTA-kernel regions (1)
+//   TRIDIAG_RAG_TMA      vector paths for ragged / pitched rows (1)
+//   TRIDIAG_TMA_PF       TMA-box L2 prefetch of the unit after next (0)
+//   TRIDIAG_SMALL_CTA    smaller warp-kernel CTAs for small batches (1)
+//   TRIDIAG_PDL          programmatic dependent launch (1)
+//   TRIDIAG_TMA          TMA CTA kernels (1)
+//   TRIDIAG_BLOCKED_MINB blocked-inner register cap (2)
+//   TRIDIAG_COL_TMA      TMA-fed column passes (1)
+//   TRIDIAG_PHASE_STAMPS per-phase clock stamps (0)
 int env_int(const char* name, int dflt) {
   const char* v = getenv(name);
   return (v && *v) ? atoi(v) : dflt;
 }
-int g_force_R = -1;
-int force_R() { if (g_force_R < 0) g_force_R = env_int("TRIDIAG_WARP_R", 0); return g_force_R; }
+
+enum Knob { kWarpR, kPrefetch, kCtaDbuf, kRagTma, kTmaPf, kSmallCta, kPdl, kTma, kBlockedMinb,
+            kColTma, kPhaseStamps, kNumKnobs };
+struct KnobDef { const char* name; int dflt; };
+constexpr KnobDef kKnobDefs[kNumKnobs] = {
+    {"TRIDIAG_WARP_R", 0},    {"TRIDIAG_PREFETCH", 2},  {"TRIDIAG_CTA_DBUF", 1},
+    {"TRIDIAG_RAG_TMA", 1},   {"TRIDIAG_TMA_PF", 0},    {"TRIDIAG_SMALL_CTA", 1},
+    {"TRIDIAG_PDL", 1},       {"TRIDIAG_TMA", 1},       {"TRIDIAG_BLOCKED_MINB", 2},
+    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}};
+std::atomic<int> g_knobs[kNumKnobs];
+std::once_flag g_knobs_once;
+std::mutex g_knobs_mu;
+
+void read_knobs() {
+  std::lock_guard<std::mutex> lk(g_knobs_mu);
+  for (int i = 0; i < kNumKnobs; ++i)
+    g_knobs[i].store(env_int(kKnobDefs[i].name, kKnobDefs[i].dflt), std::memory_order_relaxed);
+}
+int knob(Knob k) {
+  std::call_once(g_knobs_once, read_knobs);
+  return g_knobs[k].load(std::memory_order_relaxed);
+}
+int force_R() { return knob(kWarpR); }
 
 }  // namespace
 
 namespace tdg_host {
 
-int prefetch_mode() {
-  static int v = -1;
-  if (v < 0) v = env_int("TRIDIAG_PREFETCH", 2);
-  return v;
-}
-int cta_cluster_mode() { return env_int("TRIDIAG_CTA_CLUSTER", 0); }  // opt-in; read per call (A/B tests)
-int cta_dbuf_mode() {
-  static int v = -1;
-  if (v < 0) v = env_int("TRIDIAG_CTA_DBUF", 1);
-  return v;
-}
-int rag_tma_mode() { return env_int("TRIDIAG_RAG_TMA", 1); }  // read per call (A/B)
-int tma_pf_mode() { return env_int("TRIDIAG_TMA_PF", 0); }  // opt-in (measured: -1 to -8 points on rows); read per call
-int small_cta_mode() { return env_int("TRIDIAG_SMALL_CTA", 1); }  // read per call (A/B)
-int pdl_mode() {
-  static int v = -1;
-  if (v < 0) v = env_int("TRIDIAG_PDL", 1);
-  return v;
-}
-
-int tma_mode() {
-  static int v = env_int("TRIDIAG_TMA", 1);
-  return v;
-}
-int blocked_minb() {
-  static int v = env_int("TRIDIAG_BLOCKED_MINB", 2);
-  return v;
-}
+int prefetch_mode() { return knob(kPrefetch); }
+int cta_dbuf_mode() { return knob(kCtaDbuf); }
+int rag_tma_mode() { return knob(kRagTma); }
+int tma_pf_mode() { return knob(kTmaPf); }
+int small_cta_mode() { return knob(kSmallCta); }
+int pdl_mode() { return knob(kPdl); }
+int tma_mode() { return knob(kTma); }
+int blocked_minb() { return knob(kBlockedMinb); }
+int col_tma_mode() { return knob(kColTma); }
 
 // Phase stamps (diagnostic, NEXT f4): one device buffer per process, grown on
 // demand; tridiag_phase_stamps() copies the last launch's stamps back.
@@ -117,8 +133,7 @@ long long* g_stamp_dev = nullptr;
 int64_t g_stamp_cap = 0, g_stamp_len = 0;
 }  // namespace
 long long* stamp_buffer(int64_t elems) {
-  static const int on = env_int("TRIDIAG_PHASE_STAMPS", 0);
-  if (!on) return nullptr;
+  if (!knob(kPhaseStamps)) return nullptr;
   std::lock_guard<std::mutex> lk(g_stamp_mu);
   if (elems > g_stamp_cap) {
     if (g_stamp_dev) cudaFree(g_stamp_dev);
@@ -255,6 +270,16 @@ int validate(const void* a, const void* b, const void* c, const void* d, const v
   }
   *m_out = m;
   return TRIDIAG_OK;
+}
+
+// A single system (S <= 1) has no system stride, and a 1-equation system no
+// element stride: map both onto the layout the kernels expect (contiguous
+// when es == 1, else the interleaved layout with system stride 1), so the
+// element stride is always honoured.  Multi-system layouts pass unchanged.
+Layout normalise_layout(int64_t n, int64_t S, int64_t es, int64_t ss) {
+  if (n <= 1) es = 1;
+  if (S <= 1) ss = es == 1 ? n : 1;
+  return Layout{es, ss};
 }
 
 int solve_device(const void* a, const void* b, const void* c, const void* d, void* x, int64_t nr,
@@ -485,42 +510,17 @@ struct StridedPlan {
   std::vector<LargeLevel> lv;
 };
 
-// The single-pass column kernel (tridiag_colfused.cuh) replaces the passes
-// when the caller leaves bottom_n at its default and the shape allows it.
-bool col_fused_ok(int64_t np, int dtype, int algo, int64_t m, int64_t bottom_n) {
-  if (bottom_n != 0) return false;
-  const int inner = algo == TRIDIAG_CR_RD ? tdg::kRD : tdg::kPCR;
-  return dtype == TRIDIAG_F64 ? col_fused_eligible<double>(np, inner, m)
-                              : col_fused_eligible<float>(np, inner, m);
-}
-
-// Workspace of a column plan: the passes' levels, or the fused kernel's
-// survivors + counters if that is larger (either may run: the fused kernel
-// needs TMA-describable pointers, known only at the call).
+// Workspace of a column plan: the passes' reduced levels.
 size_t col_need(const StridedPlan& P, int64_t n, int64_t S, int dtype, int algo, int64_t bottom_n) {
-  size_t need = col_ws_bytes(P.lv, S, dtype);
-  const int64_t np = pad_n(n);
-  if (col_fused_ok(np, dtype, algo, P.m, bottom_n)) {
-    const size_t f = dtype == TRIDIAG_F64 ? col_fused_ws_bytes<double>(np, S) : col_fused_ws_bytes<float>(np, S);
-    need = std::max(need, f);
-  }
-  return need;
+  (void)n; (void)algo; (void)bottom_n;
+  return col_ws_bytes(P.lv, S, dtype);
 }
 
 template <typename T>
 int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
                 int64_t es, int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
-                int64_t n_last, char* ws, cudaStream_t st, bool fused) {
+                int64_t n_last, char* ws, cudaStream_t st) {
   const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
-  if (fused) {
-    cudaError_t e = cudaSuccess;
-    const int inner = algo == TRIDIAG_CR_RD ? tdg::kRD : tdg::kPCR;
-    if (col_fused<T>(a, b, c, d, x, pad_n(nr), nr, es, S, inner, m, c_pad, ws, st, &e)) {
-      if (e != cudaSuccess) return (int)e;
-      g_last_launches = 1;
-      return TRIDIAG_OK;
-    }
-  }
   struct Buf { T* a; T* b; T* c; T* d; };
   std::vector<Buf> bufs;
   char* p = ws;
@@ -646,6 +646,11 @@ const char* tridiag_status_string(int status) {
   return "unknown status";
 }
 
+void tridiag_reload_knobs(void) {
+  std::call_once(g_knobs_once, read_knobs);
+  read_knobs();
+}
+
 int64_t tridiag_max_n(int dtype, int algo) {
   if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return 0;
   switch (algo) {
@@ -681,7 +686,8 @@ int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, c
                          elem_stride, sys_stride);
   if (v != TRIDIAG_OK) return v;
   return solve_device(a, b, c, d, x, n, num_systems, dtype, algo, m,
-                      reinterpret_cast<cudaStream_t>(stream), Layout{elem_stride, sys_stride});
+                      reinterpret_cast<cudaStream_t>(stream),
+                      normalise_layout(n, num_systems, elem_stride, sys_stride));
 }
 
 int tridiag_solve_batched(const void* a, const void* b, const void* c, const void* d, void* x,
@@ -769,6 +775,7 @@ int64_t tridiag_strided_large_workspace_bytes(int64_t n, int64_t num_systems,
   if (algo < TRIDIAG_CR || algo > TRIDIAG_RD_STONE) return -1;
   if (elem_stride < 1 || sys_stride < 1) return -1;
   if (pad_n(n) > tridiag_max_n_large(dtype, algo)) return -1;
+  elem_stride = normalise_layout(n, num_systems, elem_stride, sys_stride).es;
   StridedPlan P;
   if (strided_plan(n, num_systems, elem_stride, dtype, algo, switch_level, bottom_n, switch_level, &P) !=
       TRIDIAG_OK)
@@ -789,6 +796,11 @@ int tridiag_solve_batched_strided_large(const void* a, const void* b, const void
   const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, elem_stride,
                          sys_stride, true);
   if (v != TRIDIAG_OK) return v;
+  {
+    const Layout nl = normalise_layout(n, num_systems, elem_stride, sys_stride);
+    elem_stride = nl.es;
+    sys_stride = nl.ss;
+  }
   StridedPlan P;
   const int pv = strided_plan(n, num_systems, elem_stride, dtype, algo, switch_level, bottom_n, m, &P);
   if (pv != TRIDIAG_OK) return pv;
@@ -812,16 +824,15 @@ int tridiag_solve_batched_strided_large(const void* a, const void* b, const void
                                  static_cast<double*>(x), n, num_systems, dtype, algo, P.m, P.lv,
                                  P.n_last, ws, st, num_systems > 1 ? sys_stride : n);
   }
-  const bool fused = col_fused_ok(pad_n(n), dtype, algo, P.m, bottom_n);
   if (dtype == TRIDIAG_F32)
     return solve_col_t<float>(static_cast<const float*>(a), static_cast<const float*>(b),
                               static_cast<const float*>(c), static_cast<const float*>(d),
                               static_cast<float*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
-                              P.lv, P.n_last, ws, st, fused);
+                              P.lv, P.n_last, ws, st);
   return solve_col_t<double>(static_cast<const double*>(a), static_cast<const double*>(b),
                              static_cast<const double*>(c), static_cast<const double*>(d),
                              static_cast<double*>(x), n, num_systems, elem_stride, dtype, algo, P.m,
-                             P.lv, P.n_last, ws, st, fused);
+                             P.lv, P.n_last, ws, st);
 }
 
 // Host pipeline depth: three chunk buffers on three streams, so the
@@ -859,6 +870,19 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
       for (int j = 0; j < i; ++j) cudaStreamDestroy(st[j]);
       return (int)cudaGetLastError();
     }
+  }
+  // The workspace may have been handed out by a caching allocator while work
+  // queued earlier on the legacy default stream (which orders every blocking
+  // stream) still uses it: the internal streams wait for that work first.
+  {
+    cudaEvent_t ev;
+    if (cudaEventCreateWithFlags(&ev, cudaEventDisableTiming) != cudaSuccess ||
+        cudaEventRecord(ev, cudaStreamLegacy) != cudaSuccess) {
+      for (int i = 0; i < kHostBufs; ++i) cudaStreamDestroy(st[i]);
+      return (int)cudaGetLastError();
+    }
+    for (int i = 0; i < kHostBufs; ++i) cudaStreamWaitEvent(st[i], ev, 0);
+    cudaEventDestroy(ev);
   }
   int rc = TRIDIAG_OK;
   int launches = 0;

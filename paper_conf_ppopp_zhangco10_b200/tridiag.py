@@ -64,6 +64,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_max_switch_level.restype = I64
         L.tridiag_auto_switch_level.argtypes = [I64, I, I]
         L.tridiag_auto_switch_level.restype = I
+        L.tridiag_reload_knobs.argtypes = []
+        L.tridiag_reload_knobs.restype = None
         L.tridiag_abi_version.argtypes = []
         L.tridiag_abi_version.restype = I
         L.tridiag_last_launch_count.argtypes = []
@@ -177,6 +179,11 @@ def max_switch_level(dtype, algo, n: int) -> int:
 
 def auto_switch_level(n: int, dtype, algo) -> int:
     return int(load().tridiag_auto_switch_level(int(n), _dtype_code(dtype), _algo_code(algo)))
+
+
+def reload_knobs() -> None:
+    """Re-read the TRIDIAG_* tuning knobs (diagnostic; tridiag_reload_knobs)."""
+    load().tridiag_reload_knobs()
 
 
 def abi_version() -> int:
@@ -352,7 +359,7 @@ def solve_batched_host(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, chunk_
                        workspace=None, device=None):
     """Solve a batch held in HOST memory (pinned CPU tensors for full speed).
 
-    The library pipelines chunks over two streams (H2D, solve, D2H overlap)
+    The library pipelines chunks over three streams (H2D, solve, D2H overlap)
     and returns when x is written.  ``workspace`` is a CUDA uint8 tensor of at
     least host_workspace_bytes(n, dtype, chunk_systems) bytes (allocated if None).
     """
@@ -364,6 +371,9 @@ def solve_batched_host(a, b, c, d, x=None, algo="cr_pcr", switch_level=0, chunk_
     need = host_workspace_bytes(n, d.dtype, chunk_systems)
     if workspace is None:
         workspace = torch.empty(need, dtype=torch.uint8, device=dev)
+    # the library's internal streams write the workspace: work still queued on
+    # the current (possibly non-blocking) stream must not be using it
+    torch.cuda.current_stream(workspace.device).synchronize()
     with torch.cuda.device(workspace.device):
         st = load().tridiag_solve_batched_host(
             a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(), x.data_ptr(), n, S,

@@ -204,12 +204,10 @@ def strided_large(n, S=4, es=None, ss=1, dtype=F32, algo=CR, m=0, bottom_n=0, ws
                                                              algo, m, bottom_n, ws, ws_bytes, None))
 
 
-def test_strided_large_workspace(monkeypatch):
+def test_strided_large_workspace():
     """Column passes (ADI column sweep, NEXT f1 + f2): 4 interleaved arrays of
-    n >> kin rows per pass level, 256-B aligned; with the opt-in single-kernel
-    path (TRIDIAG_COL_FUSED=1) the larger of that and its survivors + their x
-    (5 arrays of ceil(S/32)*32 systems x n/R) + counters; rows (es = 1) are
-    the large-n plan; PCR / RD and n <= 32 R need none (validation only)."""
+    n >> kin rows per pass level, 256-B aligned; rows (es = 1) are the large-n
+    plan; PCR / RD and n <= 32 R need none (validation only)."""
     assert td.column_chunk(F32) == 128 and td.column_chunk(F64) == 64
     # fp32 4096 x 4096 columns: one pass 4096 -> 256
     assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F32, CR_PCR) == 4 * 4096 * 256 * 4
@@ -218,13 +216,6 @@ def test_strided_large_workspace(monkeypatch):
         4 * 4096 * 512 * 8 + 4 * 4096 * 64 * 8
     S = 3  # ragged S: 256-B alignment of each array
     assert td.strided_large_workspace_bytes(2048, S, S, 1, F32, CR) == 4 * (-(-S * 128 * 4 // 256) * 256)
-    monkeypatch.setenv("TRIDIAG_COL_FUSED", "1")
-    counters = 1280  # 2 per 32-system group + 1, 256-B aligned (128 groups)
-    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F32, CR_PCR) == 5 * 4096 * 256 * 4 + counters
-    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F32, CR_PCR, 0, 256) == 4 * 4096 * 256 * 4
-    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F64, CR) == 5 * 4096 * 512 * 8 + counters
-    assert td.strided_large_workspace_bytes(2048, S, S, 1, F32, CR) == 5 * 32 * 128 * 4 + 256
-    monkeypatch.delenv("TRIDIAG_COL_FUSED")
     for algo in (PCR, RD):
         assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, algo) == 0
     assert td.strided_large_workspace_bytes(512, 40, 40, 1, F32, CR) == 0          # on chip

@@ -174,56 +174,50 @@ def test_column_sweep_of_a_grid_full_size_sampled():
     assert err(*sub, x[idx]).max() <= TOL[torch.float32]
 
 
-# ---------------------------------------------------------------------------
-# Single-pass column kernel (tridiag_colfused.cuh): one launch, the same CR
-# levels in the same correctly rounded operations as the passes and the
-# contiguous kernels, so bitwise equal to both.
-# ---------------------------------------------------------------------------
-FUSED_N = {torch.float32: (1024, 2048, 4096, 8192), torch.float64: (512, 1024, 2048, 4096)}
-
-
-def _passes(monkeypatch, on):
-    monkeypatch.setenv("TRIDIAG_COL_FUSED", "1" if on else "0")
 
 
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
-def test_column_fused_bitwise(dtype, monkeypatch):
-    for n in FUSED_N[dtype]:
-        for S in (36, 96):  # row pitch a multiple of 16 B (TMA)
-            rows = gen("dd", S, n, dtype, seed=n * 7 + S)
-            views = as_columns(rows)
-            for algo, m in (("cr", 0), ("cr_pcr", 0), ("cr_pcr", 2), ("cr_pcr", 8), ("cr_pcr", 32)):
-                ref = td.solve_batched(*rows, algo=algo, switch_level=m)
-                _passes(monkeypatch, True)
-                x = cols_solve(views, algo, m)
-                assert td.last_launch_count() == 1, (n, S, algo, m)
-                assert torch.equal(x.contiguous(), ref), (n, S, algo, m,
-                                                          (x.contiguous() - ref).abs().max().item())
-                _passes(monkeypatch, False)
-                xp = cols_solve(views, algo, m)
-                assert td.last_launch_count() > 1
-                assert torch.equal(xp, x)
-            assert err(*rows, x).max() <= TOL[dtype], (n, S)
-
-
-@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
-def test_column_fused_ragged_in_place_cr_rd(dtype, monkeypatch):
-    _passes(monkeypatch, True)
-    nmax = FUSED_N[dtype][-1]
-    for n, S in ((nmax - 96, 44), (FUSED_N[dtype][0] + 1, 8), (FUSED_N[dtype][1] - 5, 64)):
-        rows = gen("dd", S, n, dtype, seed=n)
-        views = as_columns(rows)
-        ref = td.solve_batched(*rows, algo="cr_pcr")
-        dcol = views[3]
-        keep = views[0].clone()
-        cols_solve(views[:3] + [dcol], "cr_pcr", x=dcol)
-        assert td.last_launch_count() == 1, n
-        assert torch.equal(dcol.contiguous(), ref), n
-        assert torch.equal(views[0], keep)
-    n = FUSED_N[dtype][2]
-    rows = gen("rdw", 40, n, dtype, seed=9)
-    views = as_columns(rows)
-    for m in (0, 8, 32):
-        x = cols_solve(views, "cr_rd", m)
-        assert td.last_launch_count() == 1, m
-        assert err(*rows, x).max() <= TOL[dtype], m
+def test_single_system_view_with_both_strides_above_one(dtype):
+    """one system whose element stride and system stride are
+    both > 1 -- e.g. a column of a grid, ``grid[:, j].unsqueeze(0)`` (strides
+    (N*N, N)) or ``t[0:1, ::2]`` -- is read and written through its element
+    stride (bitwise equal to the contiguous solve) and nothing else in the
+    parent buffer is touched, also in place (x == d)."""
+    for n in (5, 64, 500, 512, 2048, 4096):
+        if n > td.max_n(dtype, "cr"):
+            continue
+        N = n
+        rows = gen("dd", 1, n, dtype, seed=n)
+        for algo in ("cr", "cr_pcr", "pcr") if n <= td.max_n(dtype, "pcr") else ("cr", "cr_pcr"):
+            ref = td.solve_batched(*rows, algo=algo)
+            torch.cuda.synchronize()
+            views, grids = [], []
+            for t in rows:
+                g = torch.full((N, N + 3), 9.0, dtype=dtype, device="cuda")
+                g[:, 1] = t[0]
+                grids.append(g)
+                views.append(g[:, 1].unsqueeze(0))  # shape (1, n), element stride N + 3
+            assert views[0].stride()[1] == N + 3 and views[0].stride()[0] > 1
+            xg = torch.full((N, N + 3), 5.0, dtype=dtype, device="cuda")
+            xv = xg[:, 1].unsqueeze(0)
+            td.solve_batched(*views, x=xv, algo=algo)
+            torch.cuda.synchronize()
+            assert torch.equal(xv.contiguous(), ref), (n, algo)
+            mask = torch.ones_like(xg, dtype=torch.bool)
+            mask[:, 1] = False
+            assert bool((xg[mask] == 5.0).all()), (n, algo)
+            # in place through the same view
+            dv = views[3]
+            td.solve_batched(views[0], views[1], views[2], dv, x=dv, algo=algo)
+            torch.cuda.synchronize()
+            assert torch.equal(dv.contiguous(), ref), (n, algo)
+            assert bool((grids[3][mask] == 9.0).all()), (n, algo)
+        # every other element of a row: t[0:1, ::2]
+        wide = [torch.stack([t[0], torch.full_like(t[0], 3.0)], dim=1).reshape(1, 2 * n) for t in rows]
+        sv = [w[0:1, ::2] for w in wide]
+        assert sv[0].stride() == (2 * n, 2)
+        xw = torch.full((1, 2 * n), 4.0, dtype=dtype, device="cuda")
+        td.solve_batched(*sv, x=xw[0:1, ::2], algo="cr")
+        torch.cuda.synchronize()
+        assert torch.equal(xw[0, ::2], td.solve_batched(*rows, algo="cr")[0]), n
+        assert bool((xw[0, 1::2] == 4.0).all()), n

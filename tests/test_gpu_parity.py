@@ -549,26 +549,6 @@ def test_dependent_launch_chain_adi(dtype):
             assert torch.equal(out, ref), N
 
 
-@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
-def test_cluster_kernel_bitwise_equal_single_cta(dtype, monkeypatch):
-    """The opt-in 2-CTA cluster kernel for the largest on-chip systems (fp32
-    n = 8192, fp64 n = 4096; TRIDIAG_CTA_CLUSTER=1, tridiag_cta2.cuh): the
-    same CR / inner operations as the single 16-warp CTA kernel, so bitwise
-    the same x; and within the gates."""
-    n = td.max_n(dtype, "cr")
-    for S, algo, m, fam in ((37, "cr", 0, "dd"), (300, "cr_pcr", 0, "dd"), (64, "cr_pcr", 2, "dd"),
-                            (64, "cr_pcr", 16, "dd"), (64, "cr_pcr", 32, "dd"), (40, "cr_rd", 8, "rdw"),
-                            (40, "cr_rd", 32, "rdw")):
-        a, b, c, d = gen(fam, S, n, dtype, seed=S + m)
-        monkeypatch.setenv("TRIDIAG_CTA_CLUSTER", "1")
-        x1 = gpu_solve(a, b, c, d, algo, m)
-        monkeypatch.setenv("TRIDIAG_CTA_CLUSTER", "0")
-        x0 = gpu_solve(a, b, c, d, algo, m)
-        assert torch.equal(x1, x0), (S, algo, m, (x1 - x0).abs().max().item())
-        assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (S, algo, m)
-    monkeypatch.delenv("TRIDIAG_CTA_CLUSTER")
-
-
 def _residual_rel(a, b, c, d, x):
     a64, b64, c64, d64, x64 = (t.double() for t in (a, b, c, d, x))
     r = b64 * x64 - d64
@@ -621,14 +601,17 @@ def test_ragged_cta_tma_bitwise_equal_staged(dtype, monkeypatch):
             guard = torch.full((S * n + 64,), 7.0, dtype=dtype, device="cuda")
             x1 = guard[:S * n].view(S, n)
             monkeypatch.setenv("TRIDIAG_RAG_TMA", "1")
+            td.reload_knobs()
             td.solve_batched(a, b, c, d, x=x1, algo=algo, switch_level=m)
             torch.cuda.synchronize()
             monkeypatch.setenv("TRIDIAG_RAG_TMA", "0")
+            td.reload_knobs()
             x0 = gpu_solve(a, b, c, d, algo, m)
             assert torch.equal(x1, x0), (n, algo, m, (x1 - x0).abs().max().item())
             assert bool((guard[S * n:] == 7.0).all()), (n, algo, m)
             assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, algo, m)
     monkeypatch.delenv("TRIDIAG_RAG_TMA")
+    td.reload_knobs()
 
 
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
@@ -646,15 +629,18 @@ def test_ragged_warp_vector_bitwise_equal_staged(dtype, monkeypatch):
                 guard = torch.full((S * n + 64,), 7.0, dtype=dtype, device="cuda")
                 x1 = guard[:S * n].view(S, n)
                 monkeypatch.setenv("TRIDIAG_RAG_TMA", "1")
+                td.reload_knobs()
                 td.solve_batched(a, b, c, d, x=x1, algo=algo, switch_level=m)
                 torch.cuda.synchronize()
                 monkeypatch.setenv("TRIDIAG_RAG_TMA", "0")
+                td.reload_knobs()
                 x0 = gpu_solve(a, b, c, d, algo, m)
                 assert torch.equal(x1, x0), (n, S, algo)
                 assert bool((guard[S * n:] == 7.0).all()), (n, S, algo)
                 if algo != "cr_rd" or n <= 64:
                     assert err_vs_oracle(a, b, c, d, x1).max() <= TOL[dtype], (n, S, algo)
     monkeypatch.delenv("TRIDIAG_RAG_TMA")
+    td.reload_knobs()
 
 
 @pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])

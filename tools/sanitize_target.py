@@ -32,8 +32,6 @@ CASES = [
     (torch.float32, 2048, 64, "cr_pcr", 0, "column"),    # column passes, TMA-fed
     (torch.float32, 1000, 37, "cr_pcr", 0, "column"),    # column passes, direct loads, ragged
     (torch.float64, 2048, 40, "cr", 0, "column"),        # column passes fp64, two levels
-    (torch.float32, 2048, 64, "cr_pcr", 0, "column_fused"),  # single-kernel column sweep
-    (torch.float64, 1000, 40, "cr_rd", 0, "column_fused"),   # same, fp64, ragged n, RD inner
     (torch.float32, 1000, 9, "cr_pcr", 0, "contig"),     # ragged rows: TMA CTA kernel, 3-D maps
     (torch.float64, 3000, 5, "cr_rd", 0, "contig"),      # same, fp64, RD inner
     (torch.float32, 500, 37, "cr_pcr", 0, "contig"),     # ragged rows: warp kernel, 16-byte lanes
@@ -49,8 +47,7 @@ for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
         continue
     fam = "rdw" if algo in ("rd", "cr_rd") else "dd"
     a, b, c, d = inputs.generate(fam, S, n, dt, device="cuda")
-    os.environ["TRIDIAG_COL_FUSED"] = "1" if layout == "column_fused" else "0"
-    if layout in ("column", "column_fused"):
+    if layout == "column":
         views = [t.t().contiguous().t() for t in (a, b, c, d)]
     elif layout == "pitched":
         views = []
@@ -62,8 +59,6 @@ for idx, (dt, n, S, algo, m, layout) in enumerate(CASES):
         views = [a, b, c, d]
     x = td.solve_batched(*views, algo=algo, switch_level=m)
     torch.cuda.synchronize()
-    if layout == "column_fused":
-        assert td.last_launch_count() == 1, "single-kernel path did not run"
     ref = oracle.thomas(*[t.cpu().numpy() for t in (a, b, c, d)])
     e = float(np.max(oracle.normwise_error(x.contiguous().cpu().numpy(), ref)))
     tol = 1e-4 if dt == torch.float32 else 1e-10
