@@ -13,8 +13,14 @@ per-GPU workload is 256 such batches: S = 131072 systems of n = 512 (1.34 GB,
   python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
   torchrun --nproc-per-node N bench.py --gpus N ...   (weak scaling: S per GPU)
 
+  python bench.py --gpus N ...   (no torchrun: spawns the N ranks itself)
+
 --impl reference times the CPU oracle (multi-threaded fp64 Thomas, the
 paper's MT solver) on this workload; there is no reference code to install.
+
+After the timed loop the line certifies what was timed: the relative residual
+of EVERY system, the count of systems with a non-finite x, and 256 sampled
+systems per rank against the oracle (fp64 Thomas) -- "check" in the line.
 """
 from __future__ import annotations
 
@@ -53,6 +59,9 @@ def parse():
     p.add_argument("--family", default="dd")
     p.add_argument("--no-extras", action="store_true", help="skip per-algorithm table, e2e and cpu baseline")
     p.add_argument("--cpu-seconds", type=float, default=8.0, help="wall budget of the cpu_baseline leg")
+    p.add_argument("--dump-x", default="", help="save each rank's x to <path>.rank<r>.pt (harness tests)")
+    p.add_argument("--check-samples", type=int, default=256,
+                   help="systems per rank compared with the oracle after the timed loop")
     p.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
                    help="process group for the post-timing reductions (gloo: harness tests with "
                         "several ranks on one GPU)")
@@ -69,17 +78,27 @@ def measured_peak():
         return PEAK_FALLBACK_GBS, "fallback (B200_PROFILING.md)"
 
 
-def ncu_traffic(n, dtype, S):
-    """dram bytes per launch from the committed ncu --set full capture, if it
-    matches this workload (profiles/ncu_traffic.json)."""
+def ncu_traffic(kernel, n, dtype, S):
+    """DRAM bytes per launch of `kernel` (mangled name, as launched) on this
+    workload from the committed ncu --set full capture
+    (profiles/ncu_traffic.json, keyed by kernel, then by workload)."""
     path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     try:
         with open(path) as f:
             j = json.load(f)
-        key = f"{dtype}_n{n}_S{S}"
-        return j.get(key, {}).get("dram_bytes_per_launch")
+        rec = j.get(kernel, {}).get(f"{dtype}_n{n}_S{S}")
+        return rec
     except Exception:
         return None
+
+
+def demangle(name):
+    try:
+        import subprocess
+        r = subprocess.run(["c++filt"], input=name, capture_output=True, text=True, timeout=5)
+        return r.stdout.strip() or name
+    except Exception:
+        return name
 
 
 class ClockSampler:
@@ -157,73 +176,117 @@ def cpu_model():
     return "unknown"
 
 
-def cpu_baseline(n, S, dtype_t, family, budget_s):
-    """The oracle (fp64 Thomas, multi-threaded like the paper's MT solver,
-    P:L750-755) as it stands, on a bounded sample of the bench workload."""
-    import numpy as np
+CPU_CALL_SYSTEMS = 32768  # systems per oracle call, the same in cpu_baseline and --impl reference
+
+
+def _cpu_sample(n, dtype_t, family):
+    """The oracle's bounded sample of the workload: its first
+    CPU_CALL_SYSTEMS systems, as the fp64 upcast (fp32 copy for the fp32 MT
+    variant)."""
     import torch
-
-    import oracle
     from paper_conf_ppopp_zhangco10_b200 import inputs
+    return [t.to(torch.float64).numpy() for t in inputs.generate(family, CPU_CALL_SYSTEMS, n, dtype_t)]
 
-    cores = cpu_cores()
-    S_s = min(S, 32768)
-    a, b, c, d = [t.to(torch.float64).numpy() for t in inputs.generate(family, S_s, n, dtype_t)]
+
+def _time_oracle(arrs, threads, dtype, budget_s, max_reps=1000):
+    import numpy as np
+    import oracle
+    a, b, c, d = arrs
     x = np.empty_like(d)
-    oracle.thomas_mt(a, b, c, d, cores, out=x)  # warm
+    oracle.thomas_mt(a, b, c, d, threads, dtype=dtype, out=x)  # warm
     reps, t0 = 0, time.perf_counter()
     while True:
-        oracle.thomas_mt(a, b, c, d, cores, out=x)
+        oracle.thomas_mt(a, b, c, d, threads, dtype=dtype, out=x)
         reps += 1
         el = time.perf_counter() - t0
-        if el >= budget_s or reps >= 1000:
-            break
-    v = reps * S_s / el
+        if el >= budget_s or reps >= max_reps:
+            return reps, el
+
+
+def cpu_baseline(n, S, dtype_t, family, budget_s):
+    """The oracle (fp64 Thomas, multi-threaded like the paper's MT solver,
+    P:L750-755) as it stands, on a bounded sample of the bench workload; plus
+    the paper's other CPU columns (Fig 7): the MT solver in fp32
+    (the paper's precision) and single-thread Thomas ("GE") in fp64 / fp32."""
+    import numpy as np
+    cores = cpu_cores()
+    arrs = _cpu_sample(n, dtype_t, family)
+    arrs32 = [np.ascontiguousarray(v, dtype=np.float32) for v in arrs]
+    reps, el = _time_oracle(arrs, cores, np.float64, budget_s)
+    v = reps * CPU_CALL_SYSTEMS / el
+    variants = {}
+    for name, ar, thr, dt in (("fp32_mt", arrs32, cores, np.float32),
+                              ("fp64_1thread", arrs, 1, np.float64),
+                              ("fp32_1thread", arrs32, 1, np.float32)):
+        r2, e2 = _time_oracle(ar, thr, dt, max(0.5, budget_s / 4))
+        sps = r2 * CPU_CALL_SYSTEMS / e2
+        variants[name] = {"value": sps, "threads": thr, "reps": r2, "wall_s": round(e2, 3),
+                          "gbs": sps * 5 * n * (4 if dt == np.float32 else 8) / 1e9}
     return {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
-            "sample": f"{reps} x {S_s} systems of n={n} ({family}, fp64 upcast of the {str(dtype_t).replace('torch.', '')} inputs) "
-                      f"= {reps * S_s} of the workload's systems, fp64 Thomas on {cores} threads "
-                      f"({cpu_model()}), wall {el:.2f} s",
-            "gbs": v * 5 * n * (8) / 1e9}
+            "sample": f"{reps} calls x {CPU_CALL_SYSTEMS} systems of n={n} ({family}, fp64 upcast of the "
+                      f"{str(dtype_t).replace('torch.', '')} inputs) = {reps * CPU_CALL_SYSTEMS} of the "
+                      f"workload's systems, fp64 Thomas on {cores} threads ({cpu_model()}), wall {el:.2f} s",
+            "gbs": v * 5 * n * 8 / 1e9,
+            "variants": variants}
 
 
 def run_reference(args):
-    """--impl reference: the CPU oracle timed as the reference arm."""
+    """--impl reference: the CPU oracle timed as the reference arm, each step
+    one oracle call on the same CPU_CALL_SYSTEMS-system sample as cpu_baseline
+    (so the two timings of the same program agree)."""
     import numpy as np
-    import torch
-
     import oracle
-    from paper_conf_ppopp_zhangco10_b200 import inputs
+    import torch
     from paper_conf_ppopp_zhangco10_b200.partition import dist_env
 
     rank, _, world = dist_env()
     if rank != 0:
         return 0
     dt = torch.float32 if args.dtype == "f32" else torch.float64
-    n, S = args.n, args.systems
+    n = args.n
     cores = cpu_cores()
-    per_step = 2048
-    a, b, c, d = [t.to(torch.float64).numpy() for t in inputs.generate(args.family, per_step * 4, n, dt)]
-    x = np.empty((per_step, n))
-    sl = lambda v, i: v[(i % 4) * per_step:((i % 4) + 1) * per_step]
-    for i in range(args.warmup):
-        oracle.thomas_mt(sl(a, i), sl(b, i), sl(c, i), sl(d, i), cores, out=x)
+    a, b, c, d = _cpu_sample(n, dt, args.family)
+    x = np.empty_like(d)
+    for _ in range(args.warmup):
+        oracle.thomas_mt(a, b, c, d, cores, out=x)
     t0 = time.perf_counter()
-    for i in range(args.steps):
-        oracle.thomas_mt(sl(a, i), sl(b, i), sl(c, i), sl(d, i), cores, out=x)
+    for _ in range(args.steps):
+        oracle.thomas_mt(a, b, c, d, cores, out=x)
     el = time.perf_counter() - t0
-    v = args.steps * per_step / el
+    v = args.steps * CPU_CALL_SYSTEMS / el
     line = {
         "impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * el / args.steps,
         "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
         "data": "synthetic", "config": workload_config(args, 0),
         "cpu_baseline": {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
-                         "sample": f"each step: {per_step} systems of n={n} ({args.family}) of the "
-                                   f"workload, fp64 Thomas (oracle) on {cores} threads ({cpu_model()})"},
+                         "sample": f"each step: one call on {CPU_CALL_SYSTEMS} systems of n={n} "
+                                   f"({args.family}) of the workload, fp64 Thomas (oracle) on {cores} "
+                                   f"threads ({cpu_model()})"},
         "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
     return 0
+
+
+def spawn_ranks(args):
+    """--gpus N without a torchrun environment: start the N ranks here (one
+    process per GPU, the same environment torchrun would give them) and
+    return the worst exit code.  Rank 0 prints the line."""
+    import socket
+    import subprocess
+    sock = socket.socket()
+    sock.bind(("127.0.0.1", 0))
+    port = sock.getsockname()[1]
+    sock.close()
+    procs = []
+    for r in range(args.gpus):
+        env = dict(os.environ, RANK=str(r), LOCAL_RANK=str(r), WORLD_SIZE=str(args.gpus),
+                   LOCAL_WORLD_SIZE=str(args.gpus), MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+        procs.append(subprocess.Popen([sys.executable, os.path.abspath(__file__), *sys.argv[1:]],
+                                      env=env))
+    rcs = [p.wait() for p in procs]
+    return max(rcs, key=abs)
 
 
 def workload_config(args, m):
@@ -268,6 +331,69 @@ def time_solves(td, bufs, n, S, algo, m, steps, warmup, stream):
     return sum(per) / 1e3, per, launches
 
 
+def verify(td, a, b, c, d, x, samples, s0):
+    """Certify the timed result: relative residual ||Ax - d||_inf / ||d||_inf of
+    EVERY system (fp64, on the device, in chunks), systems with a non-finite
+    x, and `samples` seeded random systems against the oracle (fp64 Thomas on
+    the exact upcast; normwise error, reading R18).  Max / sum over ranks."""
+    import numpy as np
+    import torch
+    from paper_conf_ppopp_zhangco10_b200.partition import reduce_max, reduce_sum
+    S = d.shape[0]
+    res_max, nonfinite = 0.0, 0
+    step = max(1, (1 << 24) // max(1, d.shape[1]))
+    for lo in range(0, S, step):
+        hi = min(S, lo + step)
+        a64, b64, c64, d64, x64 = (t[lo:hi].double() for t in (a, b, c, d, x))
+        r = b64 * x64 - d64
+        r[:, 1:] += a64[:, 1:] * x64[:, :-1]
+        r[:, :-1] += c64[:, :-1] * x64[:, 1:]
+        rel = r.abs().amax(1) / d64.abs().amax(1).clamp_min(1e-300)
+        bad = ~torch.isfinite(x64).all(1)
+        nonfinite += int(bad.sum())
+        rel = torch.where(bad, torch.full_like(rel, float("inf")), rel)
+        res_max = max(res_max, float(rel.max()))
+    err_max = 0.0
+    k = min(samples, S)
+    if k > 0:
+        import oracle
+        idx = torch.randperm(S, generator=torch.Generator().manual_seed(20100109 + s0))[:k]
+        idx = idx.sort().values.to(d.device)
+        ha, hb, hc, hd = (t.index_select(0, idx).double().cpu().numpy() for t in (a, b, c, d))
+        ref = oracle.thomas(ha, hb, hc, hd)
+        e = oracle.normwise_error(x.index_select(0, idx).cpu().numpy(), ref)
+        err_max = float(np.max(e))
+    return {"residual_max": reduce_max(res_max), "nonfinite": int(reduce_sum(nonfinite)),
+            "error_max": reduce_max(err_max), "oracle_samples_per_rank": k,
+            "how": "after the timed loop: relative residual of every system (fp64, device); "
+                   f"{k} seeded random systems per rank vs the oracle (fp64 Thomas), normwise "
+                   "max|x - x^|/max|x^| (R18); max / sum over ranks"}
+
+
+def pcie_peaks(h, hx, reps=5):
+    """Pinned host <-> device copy rates (GB/s, best of `reps`) of one
+    buffer the size of d: the ceiling of the host-buffer path."""
+    import torch
+    dbuf = torch.empty(h.shape, dtype=h.dtype, device="cuda")
+    nb = h.numel() * h.element_size()
+    out = {}
+    for name, fn in (("h2d_gbs", lambda: dbuf.copy_(h, non_blocking=True)),
+                     ("d2h_gbs", lambda: hx.copy_(dbuf, non_blocking=True))):
+        best = float("inf")
+        for _ in range(reps):
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            torch.cuda.synchronize()
+            e0.record()
+            fn()
+            e1.record()
+            torch.cuda.synchronize()
+            best = min(best, e0.elapsed_time(e1) / 1e3)
+        out[name] = nb / best / 1e9
+    out["bytes"] = nb
+    del dbuf
+    return out
+
+
 def main():
     args = parse()
     if args.impl == "reference":
@@ -281,8 +407,16 @@ def main():
     from paper_conf_ppopp_zhangco10_b200.partition import dist_env, reduce_max
 
     rank, local, world = dist_env()
-    args.gpus = world
+    if "WORLD_SIZE" not in os.environ and args.gpus > 1:
+        return spawn_ranks(args)
+    if world != args.gpus:
+        print(f"bench.py: --gpus {args.gpus} but WORLD_SIZE={world}", file=sys.stderr)
+        return 2
     ndev = torch.cuda.device_count()
+    if args.dist_backend == "nccl" and world > ndev:
+        print(f"bench.py: {world} NCCL ranks need {world} GPUs, {ndev} visible "
+              f"(--dist-backend gloo runs several ranks on one GPU for harness tests)", file=sys.stderr)
+        return 2
     dev = local if local < ndev else local % ndev  # (>1 rank per GPU only for harness tests)
     torch.cuda.set_device(dev)
     if world > 1:
@@ -331,16 +465,25 @@ def main():
     value = total * args.steps / t_max
     ms_per_step = 1e3 * t_max / args.steps
 
+    kernels = td.last_kernel_names()
+    check = verify(td, a, b, c, d, x, args.check_samples, s0)
+    if args.dump_x:
+        torch.save({"s0": s0, "x": x.cpu()}, f"{args.dump_x}.rank{rank}.pt")
+
     peak, peak_src = measured_peak()
     kern_s = statistics.mean(per_launch_ms) / 1e3   # this rank's average launch duration
     achieved = bytes_per_step / kern_s / 1e9
-    traffic = ncu_traffic(n, args.dtype, S)
+    kname = kernels[0] if len(kernels) == 1 else None
+    prof = ncu_traffic(kname, n, args.dtype, S) if kname else None
     roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                "frac": achieved / peak, "traffic": traffic,
+                "frac": achieved / peak,
+                "traffic": prof.get("dram_bytes_per_launch") if prof else None,
+                "traffic_source": prof.get("source") if prof else "no ncu capture of this kernel on this workload",
                 "algorithmic_bytes_per_launch": bytes_per_step,
                 "peak_source": peak_src,
                 "frac_of_8TBs": achieved / 8000.0,
-                "kernel": "tdg_warp_kernel<float,16,PCR,false>" if (args.dtype == "f32" and n == 512) else "see DESIGN.md"}
+                "kernel": demangle(kname) if kname else kernels,
+                "kernel_mangled": kname}
 
     line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_per_step,
@@ -349,7 +492,11 @@ def main():
             "config": workload_config(args, m), "roofline": roofline,
             "hbm_gbs_aggregate": value * 5 * n * T / 1e9,
             "systems_in_job": total,
-            "gpu_launches": launches, "clocks": sampler.summary()}
+            "gpu_launches": launches, "clocks": sampler.summary(),
+            "check": check,
+            # the error fields SURVEY.md 8(d) / 8(c) "Metrics" name, from the check
+            "error": check["error_max"], "residual": check["residual_max"],
+            "nonfinite": check["nonfinite"]}
 
     if not args.no_extras:
         # --- e2e: host (pinned) buffers through the C ABI, copies inside the timed region
@@ -368,11 +515,20 @@ def main():
                                   chunk_systems=chunk, workspace=ws)
         e2e_local = time.perf_counter() - t0
         e2e_t = reduce_max(e2e_local)
+        pcie = pcie_peaks(hd, hx)
+        h2d_b, d2h_b = 4 * n * T * S, n * T * S
+        # full duplex: the pipeline cannot beat the slower of the two directions
+        bound_s = max(h2d_b / (pcie["h2d_gbs"] * 1e9), d2h_b / (pcie["d2h_gbs"] * 1e9))
         line["e2e"] = {"value": total * e2e_steps / e2e_t, "unit": UNIT,
-                       "h2d_bytes_per_step": 4 * n * T * S, "d2h_bytes_per_step": n * T * S,
+                       "h2d_bytes_per_step": h2d_b, "d2h_bytes_per_step": d2h_b,
+                       "h2d_gbs": h2d_b * e2e_steps / e2e_t / 1e9,
+                       "pcie_peaks": pcie,
+                       "frac_of_copy_bound": bound_s / (e2e_t / e2e_steps),
                        "how": f"tridiag_solve_batched_host on pinned host buffers, {chunk}-system "
                               f"chunks pipelined over 3 streams, {e2e_steps} steps, wall clock "
-                              f"around the blocking call, max over ranks"}
+                              f"around the blocking call, max over ranks; frac_of_copy_bound = "
+                              f"max(H2D bytes / H2D peak, D2H bytes / D2H peak) / step time, "
+                              f"peaks measured here with plain pinned cudaMemcpy"}
         del ws, ha, hb, hc, hd, hx
         # --- every algorithm on the same workload (RD family on the RD-stable POI input)
         per_algo = {}

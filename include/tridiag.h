@@ -286,6 +286,13 @@ int tridiag_abi_version(void);
  * made on this thread (0 when S == 0).  For the bench's launch count. */
 int tridiag_last_launch_count(void);
 
+/* Name (the mangled device-function symbol, as ncu prints it with
+ * --print-kernel-base mangled) of the i-th kernel launched by the last call
+ * on this thread, i = 0 .. min(tridiag_last_launch_count(), 16) - 1; NULL
+ * otherwise.  Static storage owned by the CUDA runtime.  Diagnostic: lets a
+ * benchmark name the kernel it timed and look up its profile. */
+const char* tridiag_last_kernel_name(int i);
+
 /*
  * tridiag_phase_stamps -- diagnostic (the analogue of
  * the paper's per-phase timing, Figs 8/11/13/15/16).  Only active

@@ -19,6 +19,15 @@
 namespace tdg_host {
 
 extern thread_local int g_last_launches;  // launches of the last call on this thread
+// Kernels launched by the last call on this thread, in launch order (the
+// first kMaxKernelLog; diagnostic: tridiag_last_kernel_name).
+constexpr int kMaxKernelLog = 16;
+extern thread_local const void* g_kernel_log[kMaxKernelLog];
+extern thread_local int g_kernel_log_len;
+inline void begin_call() {
+  g_last_launches = 0;
+  g_kernel_log_len = 0;
+}
 
 struct Layout {
   int64_t es, ss;  // element stride, system stride (elements)
@@ -72,6 +81,7 @@ cudaError_t launch_k(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem,
   at[0].val.programmaticStreamSerializationAllowed = 1;
   cfg.attrs = at;
   cfg.numAttrs = pdl_mode() ? 1 : 0;
+  if (g_kernel_log_len < kMaxKernelLog) g_kernel_log[g_kernel_log_len++] = reinterpret_cast<const void*>(kern);
   return cudaLaunchKernelEx(&cfg, kern, std::forward<Args>(args)...);
 }
 

@@ -18,6 +18,8 @@
 
 namespace tdg_host {
 thread_local int g_last_launches = 0;
+thread_local const void* g_kernel_log[kMaxKernelLog];
+thread_local int g_kernel_log_len = 0;
 }  // namespace tdg_host
 
 namespace {
@@ -619,6 +621,16 @@ int tridiag_abi_version(void) { return TRIDIAG_ABI_VERSION; }
 
 int tridiag_last_launch_count(void) { return g_last_launches; }
 
+const char* tridiag_last_kernel_name(int i) {
+  if (i < 0 || i >= g_kernel_log_len) return nullptr;
+  const char* name = nullptr;
+  if (cudaFuncGetName(&name, g_kernel_log[i]) != cudaSuccess) {
+    cudaGetLastError();
+    return nullptr;
+  }
+  return name;
+}
+
 int64_t tridiag_phase_stamps(int64_t* out, int64_t cap) {
   std::lock_guard<std::mutex> lk(g_stamp_mu);
   if (!g_stamp_dev || !out || cap <= 0) return 0;
@@ -680,7 +692,7 @@ int tridiag_solve_batched_strided(const void* a, const void* b, const void* c, c
                                   void* x, int64_t n, int64_t num_systems, int64_t elem_stride,
                                   int64_t sys_stride, int dtype, int algo, int switch_level,
                                   tridiag_stream_t stream) {
-  g_last_launches = 0;
+  begin_call();
   int64_t m = 0;
   const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m,
                          elem_stride, sys_stride);
@@ -729,7 +741,7 @@ int tridiag_solve_batched_large(const void* a, const void* b, const void* c, con
                                 void* x, int64_t n, int64_t num_systems, int dtype, int algo,
                                 int switch_level, int64_t bottom_n, void* workspace,
                                 int64_t workspace_bytes, tridiag_stream_t stream) {
-  g_last_launches = 0;
+  begin_call();
   int64_t m = 0;
   const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, 1, n, true);
   if (v != TRIDIAG_OK) return v;
@@ -791,7 +803,7 @@ int tridiag_solve_batched_strided_large(const void* a, const void* b, const void
                                         int algo, int switch_level, int64_t bottom_n,
                                         void* workspace, int64_t workspace_bytes,
                                         tridiag_stream_t stream) {
-  g_last_launches = 0;
+  begin_call();
   int64_t m = 0;
   const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, elem_stride,
                          sys_stride, true);
@@ -850,7 +862,7 @@ int tridiag_solve_batched_host(const void* a, const void* b, const void* c, cons
                                int64_t n, int64_t num_systems, int dtype, int algo,
                                int switch_level, void* workspace, size_t workspace_bytes,
                                int64_t chunk_systems) {
-  g_last_launches = 0;
+  begin_call();
   int64_t m = 0;
   const int v = validate(a, b, c, d, x, n, num_systems, dtype, algo, switch_level, &m, 1, n);
   if (v != TRIDIAG_OK) return v;

@@ -64,6 +64,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_max_switch_level.restype = I64
         L.tridiag_auto_switch_level.argtypes = [I64, I, I]
         L.tridiag_auto_switch_level.restype = I
+        L.tridiag_last_kernel_name.argtypes = [I]
+        L.tridiag_last_kernel_name.restype = ctypes.c_char_p
         L.tridiag_reload_knobs.argtypes = []
         L.tridiag_reload_knobs.restype = None
         L.tridiag_abi_version.argtypes = []
@@ -179,6 +181,18 @@ def max_switch_level(dtype, algo, n: int) -> int:
 
 def auto_switch_level(n: int, dtype, algo) -> int:
     return int(load().tridiag_auto_switch_level(int(n), _dtype_code(dtype), _algo_code(algo)))
+
+
+def last_kernel_names() -> list:
+    """Mangled names of the kernels the last call on this thread launched."""
+    L = load()
+    out = []
+    for i in range(min(last_launch_count(), 16)):
+        v = L.tridiag_last_kernel_name(i)
+        if v is None:
+            break
+        out.append(v.decode())
+    return out
 
 
 def reload_knobs() -> None:
