@@ -86,8 +86,13 @@ def ncu_traffic(kernel, n, dtype, S):
     try:
         with open(path) as f:
             j = json.load(f)
-        rec = j.get(kernel, {}).get(f"{dtype}_n{n}_S{S}")
-        return rec
+        # ncu's mangled names may drop the last parameter codes: match by prefix
+        for k, v in j.items():
+            if kernel.startswith(k) or k.startswith(kernel):
+                rec = v.get(f"{dtype}_n{n}_S{S}")
+                if rec:
+                    return rec
+        return None
     except Exception:
         return None
 

@@ -271,6 +271,27 @@ int64_t tridiag_max_switch_level(int dtype, int algo, int64_t n);
  * invalid arguments. */
 int tridiag_auto_switch_level(int64_t n, int dtype, int algo);
 
+/*
+ * tridiag_paper_cr -- BASELINE ONLY, not a solver to use: the paper's own
+ * GT200 kernel schedule for CR (one CTA per system, n/2 threads,
+ * the system in place in shared memory, a __syncthreads per step, the access
+ * stride doubling every step), kept so its bank conflicts and per-step times
+ * (Fig 9) can be measured on B200 beside the register-blocked
+ * kernels.  Same layout, ownership and stream semantics as
+ * tridiag_solve_batched (contiguous, x == d allowed); n a power of two,
+ * 2 <= n <= 1024; num_systems <= 2^31 - 1 (one CTA per system).
+ * mode 0: the schedule as published (correct x, G1/G2 accuracy).
+ * mode 1: the paper's timing control, every access at stride
+ *         one -- x is MEANINGLESS, for timing / ncu comparison only.
+ * With TRIDIAG_PHASE_STAMPS=1, thread 0 of each of the first 512 CTAs records
+ * clock64() after the load, each forward step, the 2x2 solve, each backward
+ * step and the store (32 slots per CTA; tridiag_phase_stamps).
+ * Returns the same status codes (mode outside {0, 1}: TRIDIAG_ERR_ALGO).
+ */
+int tridiag_paper_cr(const void* a, const void* b, const void* c, const void* d, void* x,
+                     int64_t n, int64_t num_systems, int dtype, int mode,
+                     tridiag_stream_t stream);
+
 /* Re-read the TRIDIAG_* tuning knobs from the environment (diagnostic: A/B
  * measurements and the bitwise path-equality tests).  Normally the knobs are
  * read once, on the library's first call, and never change afterwards; calling

@@ -133,4 +133,10 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
                      T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t es, int64_t S,
                      int64_t es2, int kin, T c_pad, cudaStream_t st);
 
+// The paper's own CR schedule (tridiag_paper.cuh, inst_paper.cu): Fig 9
+// baseline only.  mode 0 = in place (bank conflicts), 1 = stride-one control.
+template <typename T>
+cudaError_t paper_cr(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n, int64_t S,
+                     int mode, cudaStream_t st);
+
 }  // namespace tdg_host

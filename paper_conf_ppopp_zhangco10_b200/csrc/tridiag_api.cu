@@ -658,6 +658,33 @@ const char* tridiag_status_string(int status) {
   return "unknown status";
 }
 
+int tridiag_paper_cr(const void* a, const void* b, const void* c, const void* d, void* x,
+                     int64_t n, int64_t num_systems, int dtype, int mode, tridiag_stream_t stream) {
+  begin_call();
+  if (num_systems != 0 && (!a || !b || !c || !d || !x)) return TRIDIAG_ERR_NULL;
+  if (dtype != TRIDIAG_F32 && dtype != TRIDIAG_F64) return TRIDIAG_ERR_DTYPE;
+  if (mode != 0 && mode != 1) return TRIDIAG_ERR_ALGO;
+  if (n < 2 || !is_pow2(n)) return TRIDIAG_ERR_N;
+  if (n > 1024) return TRIDIAG_ERR_N_TOO_LARGE;
+  if (num_systems < 0 || num_systems > 0x7fffffffLL) return TRIDIAG_ERR_NUM_SYSTEMS;
+  const size_t bytes = (size_t)num_systems * (size_t)n * elem_size(dtype);
+  if (bytes > 0) {
+    if (overlaps(x, a, bytes) || overlaps(x, b, bytes) || overlaps(x, c, bytes)) return TRIDIAG_ERR_OVERLAP;
+    if (x != d && overlaps(x, d, bytes)) return TRIDIAG_ERR_OVERLAP;
+  }
+  if (num_systems == 0) return TRIDIAG_OK;
+  cudaStream_t st = reinterpret_cast<cudaStream_t>(stream);
+  const cudaError_t e =
+      dtype == TRIDIAG_F32
+          ? paper_cr<float>(static_cast<const float*>(a), static_cast<const float*>(b),
+                            static_cast<const float*>(c), static_cast<const float*>(d),
+                            static_cast<float*>(x), n, num_systems, mode, st)
+          : paper_cr<double>(static_cast<const double*>(a), static_cast<const double*>(b),
+                             static_cast<const double*>(c), static_cast<const double*>(d),
+                             static_cast<double*>(x), n, num_systems, mode, st);
+  return e == cudaSuccess ? TRIDIAG_OK : (int)e;
+}
+
 void tridiag_reload_knobs(void) {
   std::call_once(g_knobs_once, read_knobs);
   read_knobs();

@@ -64,6 +64,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_max_switch_level.restype = I64
         L.tridiag_auto_switch_level.argtypes = [I64, I, I]
         L.tridiag_auto_switch_level.restype = I
+        L.tridiag_paper_cr.argtypes = [P, P, P, P, P, I64, I64, I, I, P]
+        L.tridiag_paper_cr.restype = I
         L.tridiag_last_kernel_name.argtypes = [I]
         L.tridiag_last_kernel_name.restype = ctypes.c_char_p
         L.tridiag_reload_knobs.argtypes = []
@@ -181,6 +183,22 @@ def max_switch_level(dtype, algo, n: int) -> int:
 
 def auto_switch_level(n: int, dtype, algo) -> int:
     return int(load().tridiag_auto_switch_level(int(n), _dtype_code(dtype), _algo_code(algo)))
+
+
+def paper_cr(a, b, c, d, x=None, mode=0, stream=None):
+    """BASELINE ONLY (tridiag_paper_cr): the paper's GT200 CR schedule, one
+    CTA per system in shared memory.  mode 1 = the stride-one timing control
+    (meaningless x).  Contiguous (S, n) CUDA tensors."""
+    if x is None:
+        x = torch.empty_like(d)
+    _check_tensors([a, b, c, d, x], "cuda")
+    S, n = d.shape
+    raw = _current_raw_stream(d.device.index) if stream is None else stream.cuda_stream
+    with torch.cuda.device(d.device):
+        st = load().tridiag_paper_cr(a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                     x.data_ptr(), n, S, _dtype_code(d.dtype), int(mode), raw)
+    check(st)
+    return x
 
 
 def last_kernel_names() -> list:

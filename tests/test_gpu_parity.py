@@ -685,3 +685,30 @@ def test_gate_rejects_a_perturbed_gpu_result(dtype):
     em = err_vs_oracle(a, b, c, d, xm)
     assert em[s] > TOL[dtype], em[s]
     assert np.array_equal(np.delete(em, s), np.delete(e, s))
+
+
+# --------------------------------------------------------------------------- E5: the paper's schedule
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_paper_schedule_cr_baseline(dtype):
+    """tridiag_paper_cr (the GT200 kernel design of P:L640-696, kept as the
+    Fig 9 baseline): mode 0 solves within the G1/G2 gates for every n it
+    takes (2..1024, ragged batch, x == d in place); mode 1 (the paper's
+    stride-one timing control) runs but is not a solver."""
+    for n in (2, 4, 8, 64, 512, 1024):
+        a, b, c, d = gen("dd", RAGGED_S, n, dtype, seed=5 + n)
+        x = td.paper_cr(a, b, c, d)
+        torch.cuda.synchronize()
+        assert err_vs_oracle(a, b, c, d, x).max() <= TOL[dtype], n
+        dd = d.clone()
+        td.paper_cr(a, b, c, dd, x=dd)
+        torch.cuda.synchronize()
+        assert torch.equal(dd, x)
+        xc = td.paper_cr(a, b, c, d, mode=1)
+        torch.cuda.synchronize()
+        assert xc.shape == x.shape
+    a, b, c, d = gen("dd", 4, 2048, dtype)
+    with pytest.raises(ValueError):
+        td.paper_cr(a, b, c, d)
+    a, b, c, d = gen("dd", 4, 100, dtype)
+    with pytest.raises(ValueError):
+        td.paper_cr(a, b, c, d)

@@ -28,6 +28,9 @@ if a.layout == "cols":
 X = torch.empty_like(D)
 torch.cuda.synchronize()
 for _ in range(a.reps):
-    td.solve_batched(A, B, C, D, X, algo=a.algo, switch_level=a.m)
+    if a.algo.startswith("paper_cr"):   # the paper's schedule (Fig 9 baseline), mode 0 / 1
+        td.paper_cr(A, B, C, D, X, mode=1 if a.algo == "paper_cr1" else 0)
+    else:
+        td.solve_batched(A, B, C, D, X, algo=a.algo, switch_level=a.m)
 torch.cuda.synchronize()
 print("done", a)
