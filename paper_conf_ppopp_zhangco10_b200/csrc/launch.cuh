@@ -51,7 +51,7 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // 8 warps per CTA; a batch too small to give every SM 8 warps is spread
   // over all SMs in smaller CTAs instead (fewer warps per scheduler: the
   // latency-bound regime of the paper-sized batches, e.g. 512 x 512)
-  const bool small = vec && blocked_minb() != 1 && P >= 16 && tdg::pcr_small_cta<T, R, INNER, KB, false>();
+  const bool small = vec && blocked_minb() != 1 && P >= 4 && tdg::pcr_small_cta<T, R, INNER, KB, false>();
   int wpb = small ? 4 : 8;
   {
     const int64_t warps_needed = (S + G - 1) / G;
@@ -73,9 +73,13 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
                      reinterpret_cast<uintptr_t>(c) | reinterpret_cast<uintptr_t>(d) |
                      reinterpret_cast<uintptr_t>(x)) & 15) == 0 &&
                    rag_tma_mode();
-  auto small_kern = [] {
+  // the small-CTA PCR kernels (P = 16 or 32 lanes) with P fixed at compile time
+  auto small_kern = [&] {
     if constexpr (tdg::pcr_small_cta<T, R, INNER, KB, false>())
-      return tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true>;
+      return log2P == 5   ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 5>
+             : log2P == 4 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 4>
+             : log2P == 3 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 3>
+                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 2>;
     else
       return tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>;
   }();
@@ -219,8 +223,9 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
     }
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
+  long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
   const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode(), (int)nr,
-                                    (long long)ss);
+                                    (long long)ss, stamps);
   if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;
   *used = true;

@@ -22,6 +22,12 @@
 #ifndef TDG_BLOCKED_MINB
 #define TDG_BLOCKED_MINB 2
 #endif
+// 4-warp CTAs per SM of the small-CTA PCR kernels (pcr_small_cta): 3 for PCR
+// alone (151 registers, no spills), one more for CR+PCR with one CR level
+// (127 registers, no spills): measured 44.0 vs 41.8% and 82.7 vs 75.1% of HBM
+#ifndef TDG_PCR_SMALL_MINB
+#define TDG_PCR_SMALL_MINB 3
+#endif
 // CTAs per SM the LU-form RD kernel asks for (its three scans want ~185
 // registers: 1 CTA of 8 warps, or 2 with spills)
 #ifndef TDG_STONE_MINB
@@ -195,11 +201,15 @@ __device__ __forceinline__ void store_block16(T* p, const T (&v)[R]) {
   }
 }
 
-template <typename T, int R, int INNER, int KB, bool GEN, bool RAG = false>
+// LP >= 0: lanes per system P = 2^LP fixed at compile time (log2P ignored), so
+// every step guard of the blocked inner solvers folds and their shuffles
+// have a compile-time width (no divergent-shuffle fallbacks).
+template <typename T, int R, int INNER, int KB, bool GEN, bool RAG = false, int LP = -1>
 __device__ __forceinline__ void warp_kernel_body(
     const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c, const T* d, T* x,
-    int n, long long S, int k, int log2P, int vec, int pf, int n_real, T c_pad, long long es,
+    int n, long long S, int k, int log2P_rt, int vec, int pf, int n_real, T c_pad, long long es,
     long long ss, long long* stamps) {
+  const int log2P = LP >= 0 ? LP : log2P_rt;
   const int P = 1 << log2P;
   const int lane = threadIdx.x & 31;
   const int warp = threadIdx.x >> 5;
@@ -318,16 +328,17 @@ tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __res
 // at the 2-CTA cap); n = 64 / 128 (P < 16) are faster with the default.
 template <typename T, int R, int INNER, int KB, bool GEN>
 __host__ __device__ constexpr bool pcr_small_cta() {
-  return INNER == kPCR && (KB == 0 || KB == 1) && !GEN && sizeof(T) == 4 && R == 16;
+  return INNER == kPCR && (KB == 0 || KB == 1) && !GEN &&
+         ((sizeof(T) == 4 && R == 16) || (sizeof(T) == 8 && R == 8));
 }
-template <typename T, int R, int INNER, int KB, bool GEN, bool SMALL = false>
+template <typename T, int R, int INNER, int KB, bool GEN, bool SMALL = false, int LP = -1>
 __global__ void __launch_bounds__(SMALL ? 128 : 256,
-                                  SMALL ? 3 : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
+                                  SMALL ? (KB == 0 ? TDG_PCR_SMALL_MINB : TDG_PCR_SMALL_MINB + 1) : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
   pdl_entry();
-  warp_kernel_body<T, R, INNER, KB, GEN>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
+  warp_kernel_body<T, R, INNER, KB, GEN, false, LP>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
                                          es, ss, stamps);
 }
 
@@ -392,7 +403,7 @@ __device__ __forceinline__ void cta_inlane_forward(T (&ra)[R], T (&rb)[R], T (&r
 // and leaves x of the lane's tail in rd[R-1].
 template <typename T, int R, int W, int INNER>
 __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R], T (&rd)[R],
-                                               int k, T* heads) {
+                                               int k, T* heads, Stamp stp = Stamp()) {
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int LRH = LR > 0 ? LR : 1;
@@ -444,6 +455,7 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
         }
       }
     }
+    stp.mark(3);
     // survivors: lanes 2^kl - 1 (mod 2^kl) of every warp
     const int per_warp = 32 >> kl;
     const int msurv = W * per_warp;
@@ -473,6 +485,7 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
       else smem_rd<T>(inner, xs, msurv, ls, P, SyncCta());
     }
     __syncthreads();
+    stp.mark(4);
     // lane-level backward inside the warp
     const T xprev_warp = warp > 0 ? xs[warp * per_warp - 1] : T(0);
     T X = is_surv ? xs[j] : T(0);

@@ -105,7 +105,8 @@ template <typename T, int R, int W, int INNER, int KB, bool RAG = false>
 __global__ void __launch_bounds__(W * 32)
 tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
-                   T* x, int n, long long S, int k, int dbuf, int pf, int n_real, long long ss) {
+                   T* x, int n, long long S, int k, int dbuf, int pf, int n_real, long long ss,
+                   long long* stamps) {
   pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
@@ -154,7 +155,17 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     // race this system's reads (they are separated by the next system's
     // first barrier) and no barrier is needed at the end of a system
     T* heads = heads0 + ((dbuf > 0 && (it & 1)) ? dbuf : 0);
+    // phase stamps (diagnostic, NEXT f4): warp 0 of every CTA, first
+    // kStampSystems systems: [0] wait for the stage, [1] data arrived,
+    // [2] in-lane forward + next-warp heads, [3] lane-level forward,
+    // [4] survivors solved, [5] lane-level backward, [6] in-lane backward,
+    // [7] store issued
+    Stamp stp;
+    if (stamps != nullptr && ls < 32 && it < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + it) * kStampSlots;
+    stp.mark(0);
     mbar_wait(bar, parity);
+    stp.mark(1);
     parity ^= 1;
     T ra[R], rb[R], rc[R], rd[R];
     const int sw = (ls >> 1) & 3;
@@ -181,13 +192,16 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     cta_inlane_forward<T, R, W>(ra, rb, rc, rd, KIN, heads, [&] {
       if (ls == 0 && next < S) issue(next);
     });
+    stp.mark(2);
     T xprev;
     if constexpr (KB >= 0) {
       xprev = cta_blocked_rd<T, R, W, (KB >= 0 ? KB : 0)>(ra, rb, rc, rd, heads + W * (LR > 0 ? LR : 1) * 4);
     } else {
-      xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads);
+      xprev = cta_register_path<T, R, W, INNER>(ra, rb, rc, rd, k, heads, stp);
     }
+    stp.mark(5);
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
+    stp.mark(6);
     if constexpr (RAG) {
       T* p = x + (size_t)sys * (size_t)ss + (size_t)ls * R;
       if (ls * R + R <= n_real) {
@@ -208,6 +222,7 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     } else {
       store_block<T, R>(x + (size_t)sys * (size_t)n + (size_t)ls * R, rd, true);
     }
+    stp.mark(7);
     if (dbuf == 0) __syncthreads();  // heads / survivor regions are reused by the next system
   }
 }
