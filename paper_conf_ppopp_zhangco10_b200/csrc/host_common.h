@@ -56,6 +56,9 @@ int pdl_mode();
 int small_cta_mode();
 // L2 prefetch of the unit after the one a TMA kernel is copying (TRIDIAG_TMA_PF).
 int tma_pf_mode();
+// L2 prefetch of a CTA's first system before the dependent-launch wait
+// (TRIDIAG_PREWAIT_PF, default 1).
+int prewait_pf_mode();
 // Vector paths for ragged contiguous rows: the TMA CTA kernel with 3-D maps
 // and the warp kernel's per-lane 16-byte accesses (TRIDIAG_RAG_TMA, default 1).
 int rag_tma_mode();

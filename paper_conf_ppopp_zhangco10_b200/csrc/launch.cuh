@@ -97,7 +97,7 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   const int64_t groups = (S + (int64_t)wpb * G - 1) / ((int64_t)wpb * G);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(groups, (int64_t)device_sms(dev) * occ));
   const int pm = prefetch_mode();
-  const int pf = vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0;
+  const int pf = (vec && (pm == 1 || (pm == 2 && P == 32)) ? 1 : 0) | (prewait_pf_mode() ? 2 : 0);
   const T c_pad = INNER == tdg::kRD ? T(1) : T(0);
   long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
   const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(threads), smem, st, a, b, c, d, x, (int)n, (long long)S, k,
@@ -224,7 +224,7 @@ cudaError_t launch_cta_tma(const T* a, const T* b, const T* c, const T* d, T* x,
   }
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(S, (int64_t)device_sms(dev) * occ));
   long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
-  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, tma_pf_mode(), (int)nr,
+  const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(W * 32), smem_use, st, mA, mB, mC, mD, x, (int)n, (long long)S, k, dbuf, (tma_pf_mode() ? 1 : 0) | (prewait_pf_mode() ? 2 : 0), (int)nr,
                                     (long long)ss, stamps);
   if (lerr != cudaSuccess) return lerr;
   g_last_launches = 1;

@@ -85,19 +85,20 @@ int auto_m(int64_t n, int dtype, int algo) {
 //   TRIDIAG_BLOCKED_MINB blocked-inner register cap (2)
 //   TRIDIAG_COL_TMA      TMA-fed column passes (1)
 //   TRIDIAG_PHASE_STAMPS per-phase clock stamps (0)
+//   TRIDIAG_PREWAIT_PF   L2 prefetch of the first system before the PDL wait (1)
 int env_int(const char* name, int dflt) {
   const char* v = getenv(name);
   return (v && *v) ? atoi(v) : dflt;
 }
 
 enum Knob { kWarpR, kPrefetch, kCtaDbuf, kRagTma, kTmaPf, kSmallCta, kPdl, kTma, kBlockedMinb,
-            kColTma, kPhaseStamps, kNumKnobs };
+            kColTma, kPhaseStamps, kPrewaitPf, kNumKnobs };
 struct KnobDef { const char* name; int dflt; };
 constexpr KnobDef kKnobDefs[kNumKnobs] = {
     {"TRIDIAG_WARP_R", 0},    {"TRIDIAG_PREFETCH", 2},  {"TRIDIAG_CTA_DBUF", 1},
     {"TRIDIAG_RAG_TMA", 1},   {"TRIDIAG_TMA_PF", 0},    {"TRIDIAG_SMALL_CTA", 1},
     {"TRIDIAG_PDL", 1},       {"TRIDIAG_TMA", 1},       {"TRIDIAG_BLOCKED_MINB", 2},
-    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}};
+    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}, {"TRIDIAG_PREWAIT_PF", 1}};
 std::atomic<int> g_knobs[kNumKnobs];
 std::once_flag g_knobs_once;
 std::mutex g_knobs_mu;
@@ -126,6 +127,7 @@ int pdl_mode() { return knob(kPdl); }
 int tma_mode() { return knob(kTma); }
 int blocked_minb() { return knob(kBlockedMinb); }
 int col_tma_mode() { return knob(kColTma); }
+int prewait_pf_mode() { return knob(kPrewaitPf); }
 
 // Phase stamps (diagnostic, NEXT f4): one device buffer per process, grown on
 // demand; tridiag_phase_stamps() copies the last launch's stamps back.

@@ -201,6 +201,24 @@ __device__ __forceinline__ void store_block16(T* p, const T (&v)[R]) {
   }
 }
 
+// L2 prefetch of a warp kernel's first system group before the dependent-launch
+// wait (see tdg_cta_tma_kernel): contiguous power-of-two rows only.
+template <typename T, int R>
+__device__ __forceinline__ void warp_prefetch_first(const T* a, const T* b, const T* c, const T* d,
+                                                    int n, long long S, int log2P, int vec, int pf,
+                                                    long long ss) {
+  const int lane = threadIdx.x & 31;
+  if (!vec || !(pf & 2) || ss != n || lane >= 4) return;
+  const int wpb = blockDim.x >> 5;
+  const int G = 32 >> log2P;
+  const long long s0 = ((long long)blockIdx.x * wpb + (threadIdx.x >> 5)) * G;
+  if (s0 >= S) return;
+  const long long cnt = (S - s0) < G ? (S - s0) : G;
+  const T* base = lane == 0 ? a : lane == 1 ? b : lane == 2 ? c : d;
+  const uint32_t bytes = (uint32_t)(cnt * n * sizeof(T));
+  if (bytes % 16 == 0) prefetch_l2(base + (size_t)s0 * n, bytes);
+}
+
 // LP >= 0: lanes per system P = 2^LP fixed at compile time (log2P ignored), so
 // every step guard of the blocked inner solvers folds and their shuffles
 // have a compile-time width (no divergent-shuffle fallbacks).
@@ -231,7 +249,7 @@ __device__ __forceinline__ void warp_kernel_body(
     if (stamps != nullptr && warp == 0 && iter < kStampSystems)
       stp.p = stamps + ((long long)blockIdx.x * kStampSystems + iter) * kStampSlots;
     stp.mark(0);
-    if (pf && lane < 4 && s0 + step < S) {
+    if ((pf & 1) && lane < 4 && s0 + step < S) {
       // lanes 0..3 prefetch array a, b, c, d of this warp's next group
       const long long nx = s0 + step;
       const long long cnt = (S - nx) < G ? (S - nx) : G;
@@ -314,6 +332,7 @@ __global__ void __launch_bounds__(256)
 tdg_warp_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                 const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                 int n_real, T c_pad, long long es, long long ss, long long* stamps) {
+  if constexpr (!GEN && !RAG) warp_prefetch_first<T, R>(a, b, c, d, n, S, log2P, vec, pf, ss);
   pdl_entry();
   warp_kernel_body<T, R, INNER, KB, GEN, RAG>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
                                               es, ss, stamps);
@@ -337,6 +356,7 @@ __global__ void __launch_bounds__(SMALL ? 128 : 256,
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
+  if constexpr (!GEN) warp_prefetch_first<T, R>(a, b, c, d, n, S, LP >= 0 ? LP : log2P, vec, pf, ss);
   pdl_entry();
   warp_kernel_body<T, R, INNER, KB, GEN, false, LP>(a, b, c, d, x, n, S, k, log2P, vec, pf, n_real, c_pad,
                                          es, ss, stamps);

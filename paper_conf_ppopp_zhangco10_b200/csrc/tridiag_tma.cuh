@@ -107,12 +107,27 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
                    const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
                    T* x, int n, long long S, int k, int dbuf, int pf, int n_real, long long ss,
                    long long* stamps) {
-  pdl_entry();
   static_assert(R * sizeof(T) == 64, "TMA stage rows are 64 bytes");
   constexpr int P = 32 * W;
   constexpr int LR = ilog2c(R);
   constexpr int ROWS = P > 256 ? 256 : P;  // rows per TMA box (box dims <= 256)
   constexpr int NBOX = P / ROWS;
+  // L2 prefetch of this CTA's first system BEFORE waiting for the previous
+  // grid: a prefetch returns nothing to the SM and L2 is the point of
+  // coherence, so a later write of the previous grid still wins; it only
+  // moves the first load's DRAM latency into the previous grid's tail (the
+  // launch ramp of a back-to-back sweep).  The stage load itself follows the
+  // wait.
+  if (!RAG && (pf & 2) && threadIdx.x == 0 && blockIdx.x < S) {
+#pragma unroll
+    for (int bx = 0; bx < NBOX; ++bx) {
+      tma_prefetch_2d(&tmA, 0, (int)(blockIdx.x * P + bx * ROWS));
+      tma_prefetch_2d(&tmB, 0, (int)(blockIdx.x * P + bx * ROWS));
+      tma_prefetch_2d(&tmC, 0, (int)(blockIdx.x * P + bx * ROWS));
+      tma_prefetch_2d(&tmD, 0, (int)(blockIdx.x * P + bx * ROWS));
+    }
+  }
+  pdl_entry();
   constexpr uint32_t ARR_BYTES = P * R * sizeof(T);
   constexpr uint32_t STAGE = tma_stage_bytes<T>(R, W);
   extern __shared__ __align__(1024) unsigned char smem_raw[];
@@ -133,7 +148,7 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
         else
           tma_load_2d(stage + q * ARR_BYTES + bx * ROWS * 64, maps[q], 0,
                       (int)(sys * P + bx * ROWS), bar);
-    if (!RAG && pf && sys + gridDim.x < S) {
+    if (!RAG && (pf & 1) && sys + gridDim.x < S) {
 #pragma unroll
       for (int q = 0; q < 4; ++q)
 #pragma unroll
