@@ -222,18 +222,20 @@ int64_t tridiag_large_chunk(int dtype);
  *
  * Interleaved columns (sys_stride == 1, elem_stride >= num_systems: the ADI
  * column sweep): for CR, CR+PCR and CR+RD with
- * n_pad > bottom_n, column reduction passes of log2 R CR levels
- * -- one CTA per 32 consecutive systems x W R rows, every warp access one
- * coalesced row segment of 32 systems -- write the surviving equations, still
- * interleaved (element stride num_systems), to the workspace until at most
- * bottom_n remain; the interleaved on-chip kernel solves them; expansion
- * passes back-substitute and write x.  bottom_n: 0 = 32 R
- * (512 fp32 / 256 fp64, the interleaved kernel's capacity), else a power of
- * two in [tridiag_column_chunk(dtype) / 2, 32 R].  HBM traffic about
- * 9.6 n T per system (each level read twice) against 5 n T on chip, but every
- * access is a full row segment where the on-chip strided kernel reads 4-byte
- * pieces of 32-byte sectors.  Hybrid default m: the contiguous solve's tuned
- * m of the full size, so results are bitwise identical to
+ * n_pad > 32 R (512 fp32 / 256 fp64, the on-chip interleaved kernel's
+ * capacity), column reduction passes of log2 R CR levels -- one
+ * CTA per 32 consecutive systems x W R rows, every warp access one coalesced
+ * row segment of 32 systems -- at least one, then more until at most
+ * bottom_n equations remain; the last pass writes the surviving equations
+ * TRANSPOSED into contiguous rows of the workspace, which the row kernels
+ * solve (the same kernels as tridiag_solve_batched); expansion passes
+ * back-substitute and write x.  bottom_n: 0 = tridiag_max_n
+ * (one pass for every on-chip size), else a power of two in
+ * [tridiag_column_chunk(dtype) / 2, tridiag_max_n(dtype, CR)].  HBM traffic
+ * about 9.3 n T per system (the input is read twice) against 5 n T on chip,
+ * but every access is a full row segment where the on-chip strided kernel
+ * reads 4-byte pieces of 32-byte sectors.  Hybrid default m: the contiguous
+ * solve's tuned m of the full size, so results are bitwise identical to
  * tridiag_solve_batched on the transposed data.  PCR, RD, RD_STONE, and
  * hybrid m that the passes cannot reach, take the on-chip strided path
  * (no workspace).

@@ -127,14 +127,14 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
 
 // Interleaved-layout (ADI column sweep) passes (tridiag_colpass.cuh,
 // inst_col.cu).  which: 1 = reduction (a, b, c, d) -> (o0..o3), 2 = expansion
-// writing x to o0 from x2.  es / es2 = element strides of the input and of
-// the reduced arrays (system stride 1 for both).
+// writing x to o0 from x2.  es = element stride of the input (system stride
+// 1); row r of system s of the reduced arrays (and of x2) at r es2 + s ss2.
 template <typename T>
 int64_t col_chunk();
 template <typename T>
 cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, T* o0, T* o1,
                      T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t es, int64_t S,
-                     int64_t es2, int kin, T c_pad, cudaStream_t st);
+                     int64_t es2, int64_t ss2, int kin, T c_pad, cudaStream_t st);
 
 // The paper's own CR schedule (tridiag_paper.cuh, inst_paper.cu): Fig 9
 // baseline only.  mode 0 = in place (bank conflicts), 1 = stride-one control.

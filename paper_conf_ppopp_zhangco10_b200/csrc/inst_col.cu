@@ -49,7 +49,7 @@ bool make_col_map(CUtensorMap* m, const void* base, int64_t S, int64_t rows, int
 template <typename T>
 cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, T* o0, T* o1,
                      T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t es, int64_t S,
-                     int64_t es2, int kin, T c_pad, cudaStream_t st) {
+                     int64_t es2, int64_t ss2, int kin, T c_pad, cudaStream_t st) {
   constexpr int R = col_R<T>();
   constexpr int W = kColW;
   constexpr int LR = tdg::ilog2c(R);
@@ -72,7 +72,7 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, a, b, c, d, o0, o1,
-          o2, o3, n, n_real, es, S, es2, c_pad, tma_pf_mode());
+          o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode());
       if (lerr != cudaSuccess) return lerr;
     } else if (tma) {
       auto kern = tdg::tdg_col_expand_tma_kernel<T, R, W, K>;
@@ -81,7 +81,7 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, o0, x2, n, n_real, es,
-          S, es2, c_pad, tma_pf_mode());
+          S, es2, ss2, c_pad, tma_pf_mode());
       if (lerr != cudaSuccess) return lerr;
     } else if (which == 1) {
       auto kern = tdg::tdg_col_reduce_kernel<T, R, W, K>;
@@ -90,7 +90,7 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, a, b, c, d, o0, o1, o2, o3, n, n_real,
-          es, S, es2, c_pad);
+          es, S, es2, ss2, c_pad);
       if (lerr != cudaSuccess) return lerr;
     } else {
       auto kern = tdg::tdg_col_expand_kernel<T, R, W, K>;
@@ -98,7 +98,7 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, n, n_real, es, S,
-          es2, c_pad);
+          es2, ss2, c_pad);
       if (lerr != cudaSuccess) return lerr;
     }
     return cudaGetLastError();
@@ -117,10 +117,10 @@ template int64_t col_chunk<float>();
 template int64_t col_chunk<double>();
 template cudaError_t col_pass<float>(int, const float*, const float*, const float*, const float*,
                                      float*, float*, float*, float*, const float*, int64_t, int64_t,
-                                     int64_t, int64_t, int64_t, int, float, cudaStream_t);
+                                     int64_t, int64_t, int64_t, int64_t, int, float, cudaStream_t);
 template cudaError_t col_pass<double>(int, const double*, const double*, const double*,
                                       const double*, double*, double*, double*, double*,
                                       const double*, int64_t, int64_t, int64_t, int64_t, int64_t,
-                                      int, double, cudaStream_t);
+                                      int64_t, int, double, cudaStream_t);
 
 }  // namespace tdg_host

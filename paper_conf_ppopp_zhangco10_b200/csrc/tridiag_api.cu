@@ -446,16 +446,18 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
 
 // ---------------------------------------------------------------------------
 // Interleaved layouts with n > 32 R (the ADI column sweep, NEXT f1 + f2):
-// column reduction passes (tridiag_colpass.cuh) until the system has at most
-// col_bottom equations, the interleaved on-chip kernel on the reduced system
-// (still interleaved, element stride S, in the workspace), expansion passes.
+// column reduction passes (tridiag_colpass.cuh) -- at least one, then more
+// until the system has at most `bottom` equations (default tridiag_max_n) --
+// the last of which writes the survivors transposed into contiguous rows in
+// the workspace; the row kernels solve those reduced systems; expansion
+// passes back-substitute.
 // ---------------------------------------------------------------------------
 int64_t col_chunk_n(int dtype) { return dtype == TRIDIAG_F64 ? col_chunk<double>() : col_chunk<float>(); }
-int64_t col_bottom_max(int dtype) { return 32 * large_R(dtype); }  // interleaved kernel capacity
+int64_t col_onchip_max(int dtype) { return 32 * large_R(dtype); }  // interleaved kernel capacity
 
 int64_t resolve_col_bottom(int dtype, int64_t bottom_n) {
-  if (bottom_n == 0) return col_bottom_max(dtype);
-  if (!is_pow2(bottom_n) || bottom_n < col_chunk_n(dtype) / 2 || bottom_n > col_bottom_max(dtype)) return -1;
+  if (bottom_n == 0) return max_n_cr(dtype);
+  if (!is_pow2(bottom_n) || bottom_n < col_chunk_n(dtype) / 2 || bottom_n > max_n_cr(dtype)) return -1;
   return bottom_n;
 }
 
@@ -465,7 +467,7 @@ bool col_plan(int64_t np, int dtype, int64_t m, int64_t bottom, std::vector<Larg
   const int64_t CH = col_chunk_n(dtype);
   lv->clear();
   int64_t cur = np;
-  while (cur > bottom) {
+  while (cur > bottom || lv->empty()) {
     const int kin = std::min(LR, ilog2_64(cur / m));
     if (kin < 1 || cur % CH != 0) return false;
     lv->push_back({cur, kin});
@@ -545,13 +547,18 @@ int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr
     const T* ic = first ? c : bufs[j - 1].c;
     const T* id = first ? d : bufs[j - 1].d;
     const Buf& B = bufs[j];
+    // the last pass transposes its survivors into contiguous rows
+    const bool last = j + 1 == lv.size();
     const cudaError_t e = col_pass<T>(1, ia, ib, ic, id, B.a, B.b, B.c, B.d, nullptr, L.n,
-                                      first ? nr : L.n, first ? es : S, S, S, L.kin, c_pad, st);
+                                      first ? nr : L.n, first ? es : S, S, last ? 1 : S,
+                                      last ? n_last : 1, L.kin, c_pad, st);
     if (e != cudaSuccess) return (int)e;
     launches += 1;
   }
+  // the reduced systems, contiguous rows of n_last <= tridiag_max_n equations:
+  // the row kernels (warp / TMA CTA), in place
   const Buf& Z = bufs.back();
-  const int rc = solve_device(Z.a, Z.b, Z.c, Z.d, Z.d, n_last, S, dtype, algo, m, st, Layout{S, 1});
+  const int rc = solve_device(Z.a, Z.b, Z.c, Z.d, Z.d, n_last, S, dtype, algo, m, st, Layout{1, n_last});
   if (rc != TRIDIAG_OK) return rc;
   launches += g_last_launches;
   for (size_t jj = lv.size(); jj-- > 0;) {
@@ -562,9 +569,10 @@ int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr
     const T* ic = first ? c : bufs[jj - 1].c;
     const T* id = first ? d : bufs[jj - 1].d;
     T* ox = first ? x : bufs[jj - 1].d;
+    const bool last = jj + 1 == lv.size();
     const cudaError_t e = col_pass<T>(2, ia, ib, ic, id, ox, nullptr, nullptr, nullptr,
-                                      bufs[jj].d, L.n, first ? nr : L.n, first ? es : S, S, S,
-                                      L.kin, c_pad, st);
+                                      bufs[jj].d, L.n, first ? nr : L.n, first ? es : S, S,
+                                      last ? 1 : S, last ? n_last : 1, L.kin, c_pad, st);
     if (e != cudaSuccess) return (int)e;
     launches += 1;
   }
@@ -596,7 +604,7 @@ int strided_plan(int64_t n, int64_t S, int64_t es, int dtype, int algo, int swit
   // interleaved columns
   const int64_t bc = resolve_col_bottom(dtype, bottom_n);
   if (bc < 0) return TRIDIAG_ERR_BOTTOM_N;
-  if (np > bc && has_cr) {
+  if (np > col_onchip_max(dtype) && has_cr) {
     const int64_t m = col_m(np, dtype, algo, switch_level, bc, &P->lv, &P->n_last);
     if (m > 0) {
       P->m = m;

@@ -15,7 +15,10 @@
 //   * the reduction pass runs KIN <= log2 R in-lane CR levels (the on-chip
 //     kernels' inlane_forward_interior / inlane_tail_chain, so every update is
 //     the same correctly rounded operation sequence) and writes the n >> KIN
-//     survivors of each system, still interleaved, to the workspace.  A
+//     survivors of each system to the workspace: row r of system s at
+//     r es2 + s ss2 -- interleaved (es2 = S, ss2 = 1) for a further column
+//     pass, or transposed into contiguous rows (es2 = 1, ss2 = n >> KIN) by
+//     the last pass, whose reduced systems the fast row kernels then solve.  A
 //     warp's tail needs the next warp's head equations (shared memory); the
 //     last warp needs the next chunk's.  Each CTA walks a contiguous range of
 //     units in descending chunk order, so those are the heads the previous
@@ -27,8 +30,8 @@
 //     in-lane back-substitution.  A unit reads only its own rows,
 //     so x may alias d.
 //
-// The reduced system is solved by the interleaved on-chip kernel
-// (tridiag_ileave.cuh) once it has at most 32 R equations.
+// The last pass's reduced systems (contiguous rows, at most tridiag_max_n
+// equations) are solved by the row kernels (warp / TMA CTA kernels).
 #pragma once
 
 #include "tridiag_tma.cuh"  // mbarrier / cp.async.bulk.tensor helpers
@@ -111,7 +114,7 @@ __global__ void __launch_bounds__(W * 32, 2)
 tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                       const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                       T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
-                      long long es, long long S, long long es2, T c_pad) {
+                      long long es, long long S, long long es2, long long ss2, T c_pad) {
   pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
@@ -159,7 +162,7 @@ tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
     if (w == 0) col_put_heads<T, R, KIN>(carry + (j & 1) * HE, lane, ra, rb, rc, rd);
     inlane_tail_chain<T, R>(ra, rb, rc, rd, KIN, H);
     if (sok) {
-      const long long o = (i0 >> KIN) * es2 + s;
+      const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
       for (int q = 0; q < Q; ++q) {
         const int t = ((q + 1) << KIN) - 1;
@@ -176,7 +179,7 @@ template <typename T, int R, int W, int KIN>
 __global__ void __launch_bounds__(W * 32, 2)
 tdg_col_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                       const T* d, T* x, const T* __restrict__ x2, long long n, long long n_real,
-                      long long es, long long S, long long es2, T c_pad) {
+                      long long es, long long S, long long es2, long long ss2, T c_pad) {
   pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -195,7 +198,7 @@ tdg_col_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
     T xs[Q];
     T xprev = T(0);
     if (sok) {
-      const long long o = (i0 >> KIN) * es2 + s;
+      const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
       for (int q = 0; q < Q; ++q) xs[q] = x2[o + q * es2];
       if (i0 > 0) xprev = x2[o - es2];
@@ -278,7 +281,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                           const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                           T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
-                          long long es, long long S, long long es2, T c_pad, int pf) {
+                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf) {
   pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
@@ -353,7 +356,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (w == 0) col_put_heads<T, R, KIN>(carry + (j & 1) * HE, lane, ra, rb, rc, rd);
     inlane_tail_chain<T, R>(ra, rb, rc, rd, KIN, H);
     if (sok) {
-      const long long o = (i0 >> KIN) * es2 + s;
+      const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
       for (int q = 0; q < Q; ++q) {
         const int t = ((q + 1) << KIN) - 1;
@@ -369,7 +372,7 @@ __global__ void __launch_bounds__(W * 32, TDG_COL_EXPAND_MINB(T))
 tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                           const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
                           T* x, const T* __restrict__ x2, long long n, long long n_real,
-                          long long es, long long S, long long es2, T c_pad, int pf) {
+                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf) {
   pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -406,7 +409,7 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     T xs[Q];
     T xprev = T(0);
     if (sok) {
-      const long long o = (i0 >> KIN) * es2 + s;
+      const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
       for (int q = 0; q < Q; ++q) xs[q] = x2[o + q * es2];
       if (i0 > 0) xprev = x2[o - es2];

@@ -207,19 +207,26 @@ def strided_large(n, S=4, es=None, ss=1, dtype=F32, algo=CR, m=0, bottom_n=0, ws
 def test_strided_large_workspace():
     """Column passes (ADI column sweep, NEXT f1 + f2): 4 interleaved arrays of
     n >> kin rows per pass level, 256-B aligned; rows (es = 1) are the large-n
-    plan; PCR / RD and n <= 32 R need none (validation only)."""
+    plan; PCR / RD and n <= 32 R need none (validation only).  The last pass
+    writes the reduced systems as contiguous rows of the same size."""
     assert td.column_chunk(F32) == 128 and td.column_chunk(F64) == 64
     # fp32 4096 x 4096 columns: one pass 4096 -> 256
     assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F32, CR_PCR) == 4 * 4096 * 256 * 4
-    # fp64: 4096 -> 512 -> 64 (log2 R = 3 levels per pass, bottom 32 R = 256)
-    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F64, CR) == \
+    # fp64: one pass 4096 -> 512 (log2 R = 3 levels; the reduced rows are solved on chip)
+    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F64, CR) == 4 * 4096 * 512 * 8
+    # an explicit bottom_n below the first reduced size forces more passes
+    assert td.strided_large_workspace_bytes(4096, 4096, 4096, 1, F64, CR, 0, 256) == \
         4 * 4096 * 512 * 8 + 4 * 4096 * 64 * 8
+    # columns beyond tridiag_max_n: passes until <= tridiag_max_n (2^16 -> 4096)
+    assert td.strided_large_workspace_bytes(1 << 16, 64, 64, 1, F32, CR) == 4 * 64 * 4096 * 4
     S = 3  # ragged S: 256-B alignment of each array
     assert td.strided_large_workspace_bytes(2048, S, S, 1, F32, CR) == 4 * (-(-S * 128 * 4 // 256) * 256)
     for algo in (PCR, RD):
         assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, algo) == 0
     assert td.strided_large_workspace_bytes(512, 40, 40, 1, F32, CR) == 0          # on chip
-    assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, CR_PCR, 1024) == 0  # m beyond the passes
+    # m = 1024: one pass of one level, the row kernels run PCR on the 1024 survivors
+    assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, CR_PCR, 1024) == 4 * 40 * 1024 * 4
+    assert td.strided_large_workspace_bytes(2048, 40, 40, 1, F32, CR_PCR, 2048) == 0  # m = n: no CR level
     # rows: the large-n plan (pitched rows allowed)
     assert td.strided_large_workspace_bytes(1 << 20, 3, 1, 1 << 20, F32, CR) == \
         td.large_workspace_bytes(1 << 20, 3, F32, CR)
@@ -234,7 +241,7 @@ def test_strided_large_validation():
     assert strided_large(4096, S=40, ws_bytes=1024) == -9
     assert strided_large(4096, S=40, bottom_n=1000) == -11        # not a power of two
     assert strided_large(4096, S=40, bottom_n=32) == -11          # below column chunk / 2
-    assert strided_large(4096, S=40, bottom_n=1024) == -11        # above 32 R
+    assert strided_large(4096, S=40, bottom_n=16384) == -11       # above tridiag_max_n
     assert strided_large(4096, S=0, bottom_n=64) == 0
     assert strided_large(1 << 15, S=0) == 0                       # beyond tridiag_max_n: passes
     assert strided_large(1 << 15, S=0, algo=PCR) == -3            # PCR has no CR levels

@@ -4,8 +4,8 @@ P:L280-300, P:L656-659).
 
 Columns of a row-major (n, S) grid are S systems with element stride S and
 system stride 1.  For n > 32 R the strided-large entry point reduces them with
-column CR passes, solves the reduced (still interleaved) system on chip and
-expands.  Every CR update is the same correctly rounded operation sequence as
+column CR passes (the last one writing the reduced systems transposed, as
+contiguous rows), solves those with the row kernels and expands.  Every CR update is the same correctly rounded operation sequence as
 the contiguous kernels', so:
 
 * bitwise: x equals the contiguous solve of the transposed data (CR, CR+PCR
@@ -82,7 +82,7 @@ def test_column_passes_several_levels_and_bottom(dtype):
     rows = gen("dd", S, n, dtype, seed=7)
     views = as_columns(rows)
     ref = td.solve_batched(*rows, algo="cr")
-    for bottom in (chunk // 2, chunk, 2 * chunk):
+    for bottom in (chunk // 2, chunk, 2 * chunk, 8 * chunk):
         x = cols_solve(views, "cr", bottom=bottom)
         assert torch.equal(x.contiguous(), ref), bottom
     ref = td.solve_batched(*rows, algo="cr_pcr", switch_level=32)
@@ -147,8 +147,10 @@ def test_pcr_and_large_m_fall_back_to_on_chip_strided():
     rows = gen("dd", S, n, dtype, seed=5)
     views = as_columns(rows)
     assert td.strided_large_workspace_bytes(n, S, S, 1, dtype, "pcr") == 0
-    assert td.strided_large_workspace_bytes(n, S, S, 1, dtype, "cr_pcr", 1024) == 0
-    for algo, m in (("pcr", 0), ("cr_pcr", 1024)):
+    assert td.strided_large_workspace_bytes(n, S, S, 1, dtype, "cr_pcr", 2048) == 0
+    # m = 1024: one column pass of one CR level, PCR on the reduced rows
+    assert td.strided_large_workspace_bytes(n, S, S, 1, dtype, "cr_pcr", 1024) > 0
+    for algo, m in (("pcr", 0), ("cr_pcr", 2048), ("cr_pcr", 1024)):
         ref = td.solve_batched(*rows, algo=algo, switch_level=m)
         x = cols_solve(views, algo, m)
         assert torch.equal(x.contiguous(), ref), algo
