@@ -325,10 +325,24 @@ const char* tridiag_last_kernel_name(int i);
  *   [0] start  [1] loads + in-lane CR forward  [2] tail chain
  *   [3] lane-level CR + inner PCR/RD (or blocked inner)
  *   [4] in-lane back-substitution  [5] store issued  [6..7] unused (0)
- * Copies up to `cap` values of the last launch into host `out` (synchronous)
- * and returns how many; 0 when inactive.
+ * The TMA CTA kernel (n > 32 R) records, on warp 0:
+ *   [0] wait for the stage  [1] data arrived  [2] in-lane forward + next-warp
+ *   heads  [3] lane-level forward  [4] survivors solved  [5] lane-level
+ *   back-substitution  [6] in-lane back-substitution  [7] store issued
+ * (RD inner: [3], [4] stay 0).  The column passes: reduce [0] unit start
+ * [1] stage arrived [2] in-lane forward [3] heads + tail chain [4] survivors
+ * stored; expand [0] start [1] x2 + stage [2] forward recomputed [3] back-
+ * substituted [4] stored.  The large-n passes: reduce [0] start [1] loads +
+ * forward [2] survivors stored; expand [0] start [1] loads + forward [2]
+ * back-substituted [3] stored.  One row of 8 per CTA per unit (first 4).
+ * tridiag_paper_cr: 32 slots per CTA (see there).
+ * Copies up to `cap` values of the last launch of the last call on this
+ * thread into host `out` (synchronous) and returns how many; 0 when inactive.
  */
 int64_t tridiag_phase_stamps(int64_t* out, int64_t cap);
+/* The same for launch `launch` (0-based, < 16) of the last call on this
+ * thread (multi-launch calls: the large-n and column passes). */
+int64_t tridiag_phase_stamps_of(int launch, int64_t* out, int64_t cap);
 
 #ifdef __cplusplus
 }

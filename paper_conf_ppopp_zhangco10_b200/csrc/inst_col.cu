@@ -71,8 +71,9 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       const int occ = occupancy(dev, kern, 32 * W, smem);
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, a, b, c, d, o0, o1,
-          o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode());
+          o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode(), stamps);
       if (lerr != cudaSuccess) return lerr;
     } else if (tma) {
       auto kern = tdg::tdg_col_expand_tma_kernel<T, R, W, K>;
@@ -80,8 +81,9 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       const int occ = occupancy(dev, kern, 32 * W, smem);
       if (occ <= 0) return cudaErrorInvalidConfiguration;
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, o0, x2, n, n_real, es,
-          S, es2, ss2, c_pad, tma_pf_mode());
+          S, es2, ss2, c_pad, tma_pf_mode(), stamps);
       if (lerr != cudaSuccess) return lerr;
     } else if (which == 1) {
       auto kern = tdg::tdg_col_reduce_kernel<T, R, W, K>;

@@ -48,14 +48,16 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
     } else if (which == 1) {
       auto kern = tdg::tdg_large_reduce_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
+      long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, o1, o2, o3, hbuf, n, n_real, ss, S,
-          vec ? 1 : 0, c_pad);
+          vec ? 1 : 0, c_pad, stamps);
       if (lerr != cudaSuccess) return lerr;
     } else {
       auto kern = tdg::tdg_large_expand_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
+      long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, hbuf, n, n_real, ss, S, vec ? 1
-          : 0, c_pad);
+          : 0, c_pad, stamps);
       if (lerr != cudaSuccess) return lerr;
     }
     return cudaGetLastError();

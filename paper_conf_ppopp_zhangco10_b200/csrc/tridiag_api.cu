@@ -129,26 +129,30 @@ int blocked_minb() { return knob(kBlockedMinb); }
 int col_tma_mode() { return knob(kColTma); }
 int prewait_pf_mode() { return knob(kPrewaitPf); }
 
-// Phase stamps (diagnostic, NEXT f4): one device buffer per process, grown on
-// demand; tridiag_phase_stamps() copies the last launch's stamps back.
+// Phase stamps (diagnostic, NEXT f4): one device buffer per launch slot of a
+// call (slot = the launch's index within the call, as in the kernel log),
+// grown on demand; tridiag_phase_stamps() copies the last launch's stamps
+// back, tridiag_phase_stamps_of(i) those of launch i of the last call.
 namespace {
 std::mutex g_stamp_mu;
-long long* g_stamp_dev = nullptr;
-int64_t g_stamp_cap = 0, g_stamp_len = 0;
+long long* g_stamp_dev[kMaxKernelLog] = {};
+int64_t g_stamp_cap[kMaxKernelLog] = {}, g_stamp_len[kMaxKernelLog] = {};
 }  // namespace
 long long* stamp_buffer(int64_t elems) {
   if (!knob(kPhaseStamps)) return nullptr;
+  const int slot = g_kernel_log_len;  // index of the launch about to be made
+  if (slot >= kMaxKernelLog) return nullptr;
   std::lock_guard<std::mutex> lk(g_stamp_mu);
-  if (elems > g_stamp_cap) {
-    if (g_stamp_dev) cudaFree(g_stamp_dev);
-    g_stamp_dev = nullptr;
-    g_stamp_cap = 0;
-    if (cudaMalloc(&g_stamp_dev, elems * sizeof(long long)) != cudaSuccess) return nullptr;
-    g_stamp_cap = elems;
+  if (elems > g_stamp_cap[slot]) {
+    if (g_stamp_dev[slot]) cudaFree(g_stamp_dev[slot]);
+    g_stamp_dev[slot] = nullptr;
+    g_stamp_cap[slot] = 0;
+    if (cudaMalloc(&g_stamp_dev[slot], elems * sizeof(long long)) != cudaSuccess) return nullptr;
+    g_stamp_cap[slot] = elems;
   }
-  cudaMemset(g_stamp_dev, 0, elems * sizeof(long long));
-  g_stamp_len = elems;
-  return g_stamp_dev;
+  cudaMemset(g_stamp_dev[slot], 0, elems * sizeof(long long));
+  g_stamp_len[slot] = elems;
+  return g_stamp_dev[slot];
 }
 
 // R per lane from the plan sweep (profiles/r01_tune_plan.md): on HBM-scale
@@ -641,12 +645,18 @@ const char* tridiag_last_kernel_name(int i) {
   return name;
 }
 
-int64_t tridiag_phase_stamps(int64_t* out, int64_t cap) {
+int64_t tridiag_phase_stamps_of(int launch, int64_t* out, int64_t cap) {
+  if (launch < 0 || launch >= g_kernel_log_len || launch >= kMaxKernelLog) return 0;
   std::lock_guard<std::mutex> lk(g_stamp_mu);
-  if (!g_stamp_dev || !out || cap <= 0) return 0;
-  const int64_t len = std::min<int64_t>(cap, g_stamp_len);
-  if (cudaMemcpy(out, g_stamp_dev, len * sizeof(long long), cudaMemcpyDeviceToHost) != cudaSuccess) return 0;
+  if (!g_stamp_dev[launch] || !out || cap <= 0) return 0;
+  const int64_t len = std::min<int64_t>(cap, g_stamp_len[launch]);
+  if (cudaMemcpy(out, g_stamp_dev[launch], len * sizeof(long long), cudaMemcpyDeviceToHost) != cudaSuccess)
+    return 0;
   return len;
+}
+
+int64_t tridiag_phase_stamps(int64_t* out, int64_t cap) {
+  return tridiag_phase_stamps_of(g_kernel_log_len - 1, out, cap);
 }
 
 const char* tridiag_status_string(int status) {

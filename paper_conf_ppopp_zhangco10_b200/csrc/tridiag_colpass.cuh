@@ -34,7 +34,7 @@
 // equations) are solved by the row kernels (warp / TMA CTA kernels).
 #pragma once
 
-#include "tridiag_tma.cuh"  // mbarrier / cp.async.bulk.tensor helpers
+#include "tridiag_tma.cuh"  // mbarrier / cp.async.bulk.tensor helpers, Stamp
 
 // CTAs per SM the TMA expansion pass asks for: its 64 KB stage allows 3, which
 // caps registers at 80 -- a gain for fp64 (255 vs 267 us at 4096^2), a loss
@@ -281,7 +281,8 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                           const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                           T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
-                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf) {
+                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf,
+                          long long* stamps) {
   pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
@@ -317,6 +318,13 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
   uint32_t parity = 0;
   int j = 0;
   for (long long u = hi - 1; u >= lo; --u, ++j) {
+    // phase stamps (NEXT f4), warp 0, first kStampSystems units: [0] unit
+    // start, [1] stage arrived, [2] in-lane forward, [3] heads barrier + tail
+    // chain, [4] survivors stored
+    Stamp stp;
+    if (stamps != nullptr && threadIdx.x < 32 && j < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + j) * kStampSlots;
+    stp.mark(0);
     const long long g = u / C, ch = u - g * C;
     const long long s = g * 32 + lane;
     const bool sok = s < S;
@@ -332,6 +340,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     T ra[R], rb[R], rc[R], rd[R];
     mbar_wait(bar, parity);
     parity ^= 1;
+    stp.mark(1);
     col_read_stage<T, R, W>(stage, w, lane, ra, rb, rc, rd);
     __syncthreads();  // the stage is free: the next unit streams in during the CR levels
     if (threadIdx.x == 0 && u - 1 >= lo) {
@@ -342,6 +351,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
     inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    stp.mark(2);
     col_put_heads<T, R, KIN>(pg + w * HE, lane, ra, rb, rc, rd);
     __syncthreads();
     Heads<T, R> H;
@@ -355,6 +365,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     }
     if (w == 0) col_put_heads<T, R, KIN>(carry + (j & 1) * HE, lane, ra, rb, rc, rd);
     inlane_tail_chain<T, R>(ra, rb, rc, rd, KIN, H);
+    stp.mark(3);
     if (sok) {
       const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
@@ -364,6 +375,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
         c2[o + q * es2] = rc[t]; d2[o + q * es2] = rd[t];
       }
     }
+    stp.mark(4);
   }
 }
 
@@ -372,7 +384,8 @@ __global__ void __launch_bounds__(W * 32, TDG_COL_EXPAND_MINB(T))
 tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constant__ CUtensorMap tmB,
                           const __grid_constant__ CUtensorMap tmC, const __grid_constant__ CUtensorMap tmD,
                           T* x, const T* __restrict__ x2, long long n, long long n_real,
-                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf) {
+                          long long es, long long S, long long es2, long long ss2, T c_pad, int pf,
+                          long long* stamps) {
   pdl_entry();
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)W * R;
@@ -401,7 +414,14 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
   }
   __syncthreads();
   uint32_t parity = 0;
-  for (long long u = blockIdx.x; u < U; u += gridDim.x) {
+  int j = 0;
+  for (long long u = blockIdx.x; u < U; u += gridDim.x, ++j) {
+    // phase stamps (NEXT f4): [0] unit start, [1] survivors' x loaded + stage
+    // arrived, [2] forward levels recomputed, [3] back-substituted, [4] stored
+    Stamp stp;
+    if (stamps != nullptr && threadIdx.x < 32 && j < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + j) * kStampSlots;
+    stp.mark(0);
     const long long g = u / C, ch = u - g * C;
     const long long s = g * 32 + lane;
     const bool sok = s < S;
@@ -420,6 +440,7 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     T ra[R], rb[R], rc[R], rd[R];
     mbar_wait(bar, parity);
     parity ^= 1;
+    stp.mark(1);
     col_read_stage<T, R, W>(stage, w, lane, ra, rb, rc, rd);
     __syncthreads();
     if (threadIdx.x == 0 && u + gridDim.x < U) {
@@ -430,9 +451,11 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
     inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    stp.mark(2);
 #pragma unroll
     for (int q = 0; q < Q; ++q) rd[((q + 1) << KIN) - 1] = xs[q];
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
+    stp.mark(3);
     if (sok) {
       T* p = x + s + i0 * es;
       if (i0 + R <= n_real) {
@@ -444,6 +467,7 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
           if (i0 + t < n_real) p[t * es] = rd[t];
       }
     }
+    stp.mark(4);
   }
 }
 

@@ -21,7 +21,7 @@
 // expansion may overwrite d with x in place.
 #pragma once
 
-#include "tridiag_device.cuh"
+#include "tridiag_kernels.cuh"  // Stamp
 
 namespace tdg {
 
@@ -141,7 +141,8 @@ __global__ void __launch_bounds__(W * 32)
 tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                         T* __restrict__ c2, T* __restrict__ d2, const T* __restrict__ hbuf,
-                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad) {
+                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad,
+                        long long* stamps) {
   pdl_entry();
   constexpr int P = 32 * W;
   constexpr int NH = large_heads_elems<R>() / 4;
@@ -151,7 +152,15 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
   const long long C = n / CH;
   const long long n2 = n >> KIN;
   const int ls = threadIdx.x;
-  for (long long u = blockIdx.x; u < S * C; u += gridDim.x) {
+  int j = 0;
+  for (long long u = blockIdx.x; u < S * C; u += gridDim.x, ++j) {
+    // phase stamps (NEXT f4), warp 0, first kStampSystems units: [0] unit
+    // start, [1] loads + KIN forward levels (lanes, warps, chunk heads),
+    // [2] survivors stored
+    Stamp stp;
+    if (stamps != nullptr && ls < 32 && j < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + j) * kStampSlots;
+    stp.mark(0);
     const long long sys = u / C, ch = u - sys * C;
     const long long i0 = ch * CH + (long long)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
@@ -160,12 +169,14 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
     if (i0 + R == n) rc[R - 1] = T(0);
     const T* hrec = ch + 1 < C ? hbuf + (sys * (C - 1) + ch) * (4 * NH) : nullptr;
     large_forward<T, R, W, KIN>(ra, rb, rc, rd, hrec, sh);
+    stp.mark(1);
     const long long o = sys * n2 + (i0 >> KIN);
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
       const int t = ((q + 1) << KIN) - 1;
       a2[o + q] = ra[t]; b2[o + q] = rb[t]; c2[o + q] = rc[t]; d2[o + q] = rd[t];
     }
+    stp.mark(2);
     __syncthreads();  // sh is reused by the next unit
   }
 }
@@ -176,7 +187,8 @@ template <typename T, int R, int W, int KIN>
 __global__ void __launch_bounds__(W * 32)
 tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, const T* __restrict__ x2, const T* __restrict__ hbuf,
-                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad) {
+                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad,
+                        long long* stamps) {
   pdl_entry();
   constexpr int P = 32 * W;
   constexpr int NH = large_heads_elems<R>() / 4;
@@ -186,7 +198,14 @@ tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
   const long long C = n / CH;
   const long long n2 = n >> KIN;
   const int ls = threadIdx.x;
-  for (long long u = blockIdx.x; u < S * C; u += gridDim.x) {
+  int j = 0;
+  for (long long u = blockIdx.x; u < S * C; u += gridDim.x, ++j) {
+    // phase stamps (NEXT f4): [0] unit start, [1] loads + KIN forward levels
+    // recomputed, [2] back-substituted, [3] stored
+    Stamp stp;
+    if (stamps != nullptr && ls < 32 && j < kStampSystems)
+      stp.p = stamps + ((long long)blockIdx.x * kStampSystems + j) * kStampSlots;
+    stp.mark(0);
     const long long sys = u / C, ch = u - sys * C;
     const long long i0 = ch * CH + (long long)ls * R;
     T ra[R], rb[R], rc[R], rd[R];
@@ -201,9 +220,11 @@ tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
     const T xprev = i0 > 0 ? x2[o - 1] : T(0);
     const T* hrec = ch + 1 < C ? hbuf + (sys * (C - 1) + ch) * (4 * NH) : nullptr;
     large_forward<T, R, W, KIN>(ra, rb, rc, rd, hrec, sh);
+    stp.mark(1);
 #pragma unroll
     for (int q = 0; q < Q; ++q) rd[((q + 1) << KIN) - 1] = xs[q];
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
+    stp.mark(2);
     T* xb = x + sys * ss;
     if (vec) {
       store_block<T, R>(xb + i0, rd, true);
@@ -212,6 +233,7 @@ tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
       for (int t = 0; t < R; ++t)
         if (i0 + t < n_real) xb[i0 + t] = rd[t];
     }
+    stp.mark(3);
     __syncthreads();
   }
 }

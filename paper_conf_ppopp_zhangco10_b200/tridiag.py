@@ -76,6 +76,8 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
         L.tridiag_last_launch_count.restype = I
         L.tridiag_phase_stamps.argtypes = [P, I64]
         L.tridiag_phase_stamps.restype = I64
+        L.tridiag_phase_stamps_of.argtypes = [I, P, I64]
+        L.tridiag_phase_stamps_of.restype = I64
         L.tridiag_solve_batched_large.argtypes = [P, P, P, P, P, I64, I64, I, I, I, I64, P, I64, P]
         L.tridiag_solve_batched_large.restype = I
         L.tridiag_large_workspace_bytes.argtypes = [I64, I64, I, I, I, I64]
@@ -226,12 +228,17 @@ def last_launch_count() -> int:
     return int(load().tridiag_last_launch_count())
 
 
-def phase_stamps(cap: int = 1 << 20):
-    """Per-phase clock64() stamps of the last launch (TRIDIAG_PHASE_STAMPS=1
-    only), as an (rows, 8) int64 tensor; empty when inactive."""
+def phase_stamps(cap: int = 1 << 20, launch: int = -1, width: int = 8):
+    """Per-phase clock64() stamps (TRIDIAG_PHASE_STAMPS=1 only) of the last
+    launch of the last call (launch=-1) or of launch `launch` of it, as a
+    (rows, width) int64 tensor; empty when inactive."""
     buf = torch.zeros(cap, dtype=torch.int64)
-    n = int(load().tridiag_phase_stamps(buf.data_ptr(), cap))
-    return buf[: n - n % 8].view(-1, 8)
+    L = load()
+    if launch < 0:
+        n = int(L.tridiag_phase_stamps(buf.data_ptr(), cap))
+    else:
+        n = int(L.tridiag_phase_stamps_of(int(launch), buf.data_ptr(), cap))
+    return buf[: n - n % width].view(-1, width)
 
 
 def solve_batched_raw(a_ptr, b_ptr, c_ptr, d_ptr, x_ptr, n, num_systems, dtype, algo,

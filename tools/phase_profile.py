@@ -60,6 +60,43 @@ def run_cta(dts, n, S, algo, m):
     return out
 
 
+PASS_PHASES = {
+    "col_reduce": ["wait for the TMA stage", "in-lane CR forward", "heads barrier + tail chain",
+                   "survivor stores"],
+    "col_expand": ["x2 loads + wait for the TMA stage", "in-lane forward (recomputed)",
+                   "in-lane back-substitution", "x stores"],
+    "large_reduce": ["loads + KIN forward levels (lanes, warps, chunk heads)", "survivor stores"],
+    "large_expand": ["loads + KIN forward levels (recomputed)", "in-lane back-substitution",
+                     "x stores"],
+}
+
+
+def run_passes(dts, n, S, layout, algo="cr_pcr"):
+    """Per-launch phase cycles of the multi-launch paths (column passes, large n)."""
+    dt = torch.float32 if dts == "f32" else torch.float64
+    g = inputs.generate("dd", S, n, dt, device="cuda")
+    if layout == "cols":
+        g = [t.t().contiguous().t() for t in g]
+    for _ in range(2):
+        td.solve_batched(*g, algo=algo)
+    torch.cuda.synchronize()
+    out = {"dtype": dts, "n": n, "S": S, "layout": layout, "algo": algo, "launches": []}
+    for i, k in enumerate(td.last_kernel_names()):
+        kind = next((key for key in PASS_PHASES if key in k), None)
+        st = td.phase_stamps(launch=i).double()
+        st = st[st[:, 0] > 0]
+        rec = {"launch": i, "kernel": k[:60], "units": int(st.shape[0])}
+        if kind is not None and st.shape[0] > 0:
+            names = PASS_PHASES[kind]
+            dl = (st[:, 1:len(names) + 1] - st[:, 0:len(names)]).mean(0).tolist()
+            tot = sum(dl)
+            rec["pass"] = kind
+            rec["cycles_per_unit"] = tot
+            rec["phases"] = {nm: {"cycles": v, "share": v / tot} for nm, v in zip(names, dl)}
+        out["launches"].append(rec)
+    return out
+
+
 def run(dts, n, S, algo, m):
     dt = torch.float32 if dts == "f32" else torch.float64
     fam = "poi" if algo in ("rd", "cr_rd") else "dd"
@@ -90,3 +127,7 @@ if __name__ == "__main__":
     if which in ("all", "cta"):
         for cfg in CTA_CONFIGS:
             print(json.dumps(run_cta(*cfg)), flush=True)
+    if which in ("all", "passes"):
+        for cfg in (("f32", 4096, 4096, "cols"), ("f64", 4096, 4096, "cols"),
+                    ("f32", 1 << 20, 64, "rows"), ("f64", 1 << 20, 32, "rows")):
+            print(json.dumps(run_passes(*cfg)), flush=True)
