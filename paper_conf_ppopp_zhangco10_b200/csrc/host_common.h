@@ -59,6 +59,8 @@ int tma_pf_mode();
 // L2 prefetch of a CTA's first system before the dependent-launch wait
 // (TRIDIAG_PREWAIT_PF, default 1).
 int prewait_pf_mode();
+// Column expansion pass unit order: 1 = chunk-major (TRIDIAG_COL_ORDER).
+int col_order_mode();
 // Vector paths for ragged contiguous rows: the TMA CTA kernel with 3-D maps
 // and the warp kernel's per-lane 16-byte accesses (TRIDIAG_RAG_TMA, default 1).
 int rag_tma_mode();

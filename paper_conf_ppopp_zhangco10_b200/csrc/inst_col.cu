@@ -83,7 +83,7 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
       long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, o0, x2, n, n_real, es,
-          S, es2, ss2, c_pad, tma_pf_mode(), stamps);
+          S, es2, ss2, c_pad, tma_pf_mode() | (col_order_mode() ? 4 : 0), stamps);
       if (lerr != cudaSuccess) return lerr;
     } else if (which == 1) {
       auto kern = tdg::tdg_col_reduce_kernel<T, R, W, K>;

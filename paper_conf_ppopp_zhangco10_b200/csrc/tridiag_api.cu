@@ -86,19 +86,20 @@ int auto_m(int64_t n, int dtype, int algo) {
 //   TRIDIAG_COL_TMA      TMA-fed column passes (1)
 //   TRIDIAG_PHASE_STAMPS per-phase clock stamps (0)
 //   TRIDIAG_PREWAIT_PF   L2 prefetch of the first system before the PDL wait (1)
+//   TRIDIAG_COL_ORDER    chunk-major unit order of the column expansion pass (1)
 int env_int(const char* name, int dflt) {
   const char* v = getenv(name);
   return (v && *v) ? atoi(v) : dflt;
 }
 
 enum Knob { kWarpR, kPrefetch, kCtaDbuf, kRagTma, kTmaPf, kSmallCta, kPdl, kTma, kBlockedMinb,
-            kColTma, kPhaseStamps, kPrewaitPf, kNumKnobs };
+            kColTma, kPhaseStamps, kPrewaitPf, kColOrder, kNumKnobs };
 struct KnobDef { const char* name; int dflt; };
 constexpr KnobDef kKnobDefs[kNumKnobs] = {
     {"TRIDIAG_WARP_R", 0},    {"TRIDIAG_PREFETCH", 2},  {"TRIDIAG_CTA_DBUF", 1},
     {"TRIDIAG_RAG_TMA", 1},   {"TRIDIAG_TMA_PF", 0},    {"TRIDIAG_SMALL_CTA", 1},
     {"TRIDIAG_PDL", 1},       {"TRIDIAG_TMA", 1},       {"TRIDIAG_BLOCKED_MINB", 2},
-    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}, {"TRIDIAG_PREWAIT_PF", 1}};
+    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}, {"TRIDIAG_PREWAIT_PF", 1}, {"TRIDIAG_COL_ORDER", 1}};
 std::atomic<int> g_knobs[kNumKnobs];
 std::once_flag g_knobs_once;
 std::mutex g_knobs_mu;
@@ -128,6 +129,7 @@ int tma_mode() { return knob(kTma); }
 int blocked_minb() { return knob(kBlockedMinb); }
 int col_tma_mode() { return knob(kColTma); }
 int prewait_pf_mode() { return knob(kPrewaitPf); }
+int col_order_mode() { return knob(kColOrder); }
 
 // Phase stamps (diagnostic, NEXT f4): one device buffer per launch slot of a
 // call (slot = the launch's index within the call, as in the kernel log),

@@ -397,13 +397,23 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
   const long long C = n / CH;
   const long long U = ((S + 31) >> 5) * C;
   const CUtensorMap* maps[4] = {&tmA, &tmB, &tmC, &tmD};
+  // unit order: pf & 4 = chunk-major (the CTAs active at one time read the
+  // same rows of consecutive 32-system groups: long contiguous row spans),
+  // else group-major
+  const long long GT = (S + 31) >> 5;
+  const bool cmaj = (pf & 4) != 0;
+  auto unit = [&](long long uu, long long& gg, long long& cc) {
+    if (cmaj) { cc = uu / GT; gg = uu - cc * GT; } else { gg = uu / C; cc = uu - gg * C; }
+  };
   auto issue = [&](long long uu) {
-    const long long gg = uu / C, cc = uu - gg * C;
+    long long gg, cc;
+    unit(uu, gg, cc);
     mbar_arrive_expect_tx(bar, 4 * ARR);
 #pragma unroll
     for (int q = 0; q < 4; ++q) tma_load_2d(stage + q * ARR, maps[q], (int)(gg * 32), (int)(cc * CH), bar);
-    if (pf && uu + gridDim.x < U) {  // the unit after: toward L2
-      const long long u2 = uu + gridDim.x, g2 = u2 / C, c2 = u2 - g2 * C;
+    if ((pf & 1) && uu + gridDim.x < U) {  // the unit after: toward L2
+      long long g2, c2;
+      unit(uu + gridDim.x, g2, c2);
 #pragma unroll
       for (int q = 0; q < 4; ++q) tma_prefetch_2d(maps[q], (int)(g2 * 32), (int)(c2 * CH));
     }
@@ -422,7 +432,8 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (stamps != nullptr && threadIdx.x < 32 && j < kStampSystems)
       stp.p = stamps + ((long long)blockIdx.x * kStampSystems + j) * kStampSlots;
     stp.mark(0);
-    const long long g = u / C, ch = u - g * C;
+    long long g, ch;
+    unit(u, g, ch);
     const long long s = g * 32 + lane;
     const bool sok = s < S;
     const long long i0 = ch * CH + (long long)w * R;
