@@ -70,10 +70,17 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       const size_t smem = tdg::col_reduce_tma_smem<T, R, W>();
       const int occ = occupancy(dev, kern, 32 * W, smem);
       if (occ <= 0) return cudaErrorInvalidConfiguration;
-      const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      // row-aligned pieces when every group gets at least one CTA
+      const int64_t groups = (S + 31) / 32, C = n / CH;
+      int pieces = 0;
+      if (col_order_mode() && groups <= grid) {
+        pieces = (int)std::min<int64_t>(C, grid / groups);
+        grid = groups * pieces;
+      }
       long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
       const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, a, b, c, d, o0, o1,
-          o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode(), stamps);
+          o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode(), stamps, pieces);
       if (lerr != cudaSuccess) return lerr;
     } else if (tma) {
       auto kern = tdg::tdg_col_expand_tma_kernel<T, R, W, K>;

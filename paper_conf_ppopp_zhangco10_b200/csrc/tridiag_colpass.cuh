@@ -282,7 +282,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
                           const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
                           T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
                           long long es, long long S, long long es2, long long ss2, T c_pad, int pf,
-                          long long* stamps) {
+                          long long* stamps, int pieces) {
   pdl_entry();
   constexpr int HE = col_heads_elems<T, R>();
   constexpr int Q = R >> KIN;
@@ -296,8 +296,20 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   const long long C = n / CH;
   const long long U = ((S + 31) >> 5) * C;
-  const long long lo = (long long)blockIdx.x * U / gridDim.x;
-  const long long hi = ((long long)blockIdx.x + 1) * U / gridDim.x;
+  // pieces > 0 (gridDim = groups x pieces): CTA c walks chunk range
+  // [p C / pieces, (p + 1) C / pieces) of group c % groups, p = c / groups, so
+  // the CTAs active together read the same rows of consecutive groups (long
+  // contiguous row spans); else a contiguous split of the group-major units
+  long long lo, hi;
+  if (pieces > 0) {
+    const long long GT = (S + 31) >> 5;
+    const long long gq = blockIdx.x % GT, p = blockIdx.x / GT;
+    lo = gq * C + p * C / pieces;
+    hi = gq * C + (p + 1) * C / pieces;
+  } else {
+    lo = (long long)blockIdx.x * U / gridDim.x;
+    hi = ((long long)blockIdx.x + 1) * U / gridDim.x;
+  }
   const CUtensorMap* maps[4] = {&tmA, &tmB, &tmC, &tmD};
   auto issue = [&](long long uu) {
     const long long gg = uu / C, cc = uu - gg * C;
