@@ -28,6 +28,9 @@
 #ifndef TDG_PCR_SMALL_MINB
 #define TDG_PCR_SMALL_MINB 3
 #endif
+#ifndef TDG_PCR_SMALL_MINB_K1
+#define TDG_PCR_SMALL_MINB_K1 4
+#endif
 // CTAs per SM the LU-form RD kernel asks for (its three scans want ~185
 // registers: 1 CTA of 8 warps, or 2 with spills)
 #ifndef TDG_STONE_MINB
@@ -352,7 +355,7 @@ __host__ __device__ constexpr bool pcr_small_cta() {
 }
 template <typename T, int R, int INNER, int KB, bool GEN, bool SMALL = false, int LP = -1>
 __global__ void __launch_bounds__(SMALL ? 128 : 256,
-                                  SMALL ? (KB == 0 ? TDG_PCR_SMALL_MINB : TDG_PCR_SMALL_MINB + 1) : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
+                                  SMALL ? (KB == 0 ? TDG_PCR_SMALL_MINB : TDG_PCR_SMALL_MINB_K1) : (R >= 8 && INNER != kSTONE) ? TDG_BLOCKED_MINB : TDG_STONE_MINB)
 tdg_warp_blocked_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* d, T* x, int n, long long S, int k, int log2P, int vec, int pf,
                         int n_real, T c_pad, long long es, long long ss, long long* stamps) {
