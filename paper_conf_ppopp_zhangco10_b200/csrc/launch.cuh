@@ -52,6 +52,8 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
   // over all SMs in smaller CTAs instead (fewer warps per scheduler: the
   // latency-bound regime of the paper-sized batches, e.g. 512 x 512)
   const bool small = vec && blocked_minb() != 1 && P >= 4 && tdg::pcr_small_cta<T, R, INNER, KB, false>();
+  // compile-time P: the small-CTA PCR kernels and the LU-form RD kernel
+  const bool lp_fixed = small || (vec && blocked_minb() != 1 && P >= 4 && INNER == tdg::kSTONE);
   int wpb = small ? 4 : 8;
   {
     const int64_t warps_needed = (S + G - 1) / G;
@@ -73,13 +75,18 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
                      reinterpret_cast<uintptr_t>(c) | reinterpret_cast<uintptr_t>(d) |
                      reinterpret_cast<uintptr_t>(x)) & 15) == 0 &&
                    rag_tma_mode();
-  // the small-CTA PCR kernels (P = 16 or 32 lanes) with P fixed at compile time
+  // the small-CTA PCR kernels and the LU-form RD kernel with P fixed at compile time
   auto small_kern = [&] {
     if constexpr (tdg::pcr_small_cta<T, R, INNER, KB, false>())
       return log2P == 5   ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 5>
              : log2P == 4 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 4>
              : log2P == 3 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 3>
                           : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, true, 2>;
+    else if constexpr (INNER == tdg::kSTONE)  // LU-form RD: P fixed at compile time too
+      return log2P == 5   ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, false, 5>
+             : log2P == 4 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, false, 4>
+             : log2P == 3 ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, false, 3>
+                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false, false, 2>;
     else
       return tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>;
   }();
@@ -87,7 +94,7 @@ cudaError_t launch_warp_k(const T* a, const T* b, const T* c, const T* d, T* x, 
             : (KB < 0 && vec) ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
             : (KB < 0)        ? tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>
             : vec ? (blocked_minb() == 1 ? tdg::tdg_warp_kernel<T, R, INNER, KB, false>
-                     : small             ? small_kern
+                     : lp_fixed          ? small_kern
                                          : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, false>)
                   : tdg::tdg_warp_blocked_kernel<T, R, INNER, KB, true>;
   const size_t tiles = (vec || rag) ? 0 : (((size_t)wpb * 4 * tdg::warp_tile_elems<T, R>() * sizeof(T) + 15) & ~size_t(15));
