@@ -223,3 +223,23 @@ def test_single_system_view_with_both_strides_above_one(dtype):
         torch.cuda.synchronize()
         assert torch.equal(xw[0, ::2], td.solve_batched(*rows, algo="cr")[0]), n
         assert bool((xw[0, 1::2] == 4.0).all()), n
+
+
+@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
+def test_column_unit_order_is_bitwise_neutral(dtype, monkeypatch):
+    """The row-aligned unit orders of the column passes (TRIDIAG_COL_ORDER=1,
+    default: chunk-major expansion, grid = groups x pieces reduction) change
+    only which CTA computes which unit: bitwise the same x as the group-major
+    order, for full and ragged 32-system groups and several grid shapes."""
+    for n, S in ((4096 if dtype == torch.float32 else 2048, 100), (1024, 33), (2048, 600)):
+        rows = gen("dd", S, n, dtype, seed=n + S)
+        views = as_columns(rows)
+        out = {}
+        for v in ("1", "0"):
+            monkeypatch.setenv("TRIDIAG_COL_ORDER", v)
+            td.reload_knobs()
+            out[v] = cols_solve(views, "cr_pcr").contiguous()
+        monkeypatch.delenv("TRIDIAG_COL_ORDER")
+        td.reload_knobs()
+        assert torch.equal(out["1"], out["0"]), (n, S)
+        assert torch.equal(out["1"], td.solve_batched(*rows, algo="cr_pcr")), (n, S)

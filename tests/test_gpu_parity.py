@@ -712,3 +712,24 @@ def test_paper_schedule_cr_baseline(dtype):
     a, b, c, d = gen("dd", 4, 100, dtype)
     with pytest.raises(ValueError):
         td.paper_cr(a, b, c, d)
+
+
+def test_prewait_prefetch_is_bitwise_neutral(monkeypatch):
+    """The L2 prefetch of a CTA's first system before the dependent-launch
+    wait (TRIDIAG_PREWAIT_PF) moves no data into registers: identical x with
+    it on and off, including a dependent chain of launches (x of one solve is
+    the d of the next, so a stale read would show)."""
+    for dtype, n, S in ((torch.float32, 512, 4000), (torch.float32, 4096, 300), (torch.float64, 2048, 300)):
+        a, b, c, d = gen("dd", S, n, dtype, seed=n)
+        res = {}
+        for v in ("1", "0"):
+            monkeypatch.setenv("TRIDIAG_PREWAIT_PF", v)
+            td.reload_knobs()
+            x = d.clone()
+            for _ in range(4):
+                td.solve_batched(a, b, c, x, x=x, algo="cr_pcr")   # in place, back to back
+            torch.cuda.synchronize()
+            res[v] = x
+        monkeypatch.delenv("TRIDIAG_PREWAIT_PF")
+        td.reload_knobs()
+        assert torch.equal(res["1"], res["0"]), (n, S)
