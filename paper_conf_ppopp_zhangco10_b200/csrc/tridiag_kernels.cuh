@@ -444,7 +444,8 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
       if (l <= kl) {
         const int sg = 1 << (l - 1);
         const int md = lane & (2 * sg - 1);
-        if (md == sg - 1) B = Arith<T>::rcp(B);
+        const T rcB = rcp1(B);  // every lane (no divergent slow-path branch)
+        if (md == sg - 1) B = rcB;
         const T la = shup(A, sg, 32), lb = shup(B, sg, 32), lc = shup(C, sg, 32), ld = shup(D, sg, 32);
         const T ha = shdn(A, sg, 32), hb = shdn(B, sg, 32), hc = shdn(C, sg, 32), hd = shdn(D, sg, 32);
         if (md == 2 * sg - 1 && lane != 31) cr_unit(A, B, C, D, la, lb, lc, ld, ha, hb, hc, hd);
