@@ -138,7 +138,7 @@ tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
       // first unit of this CTA: the next chunk's heads from its first R rows
       T ha[R], hb[R], hc[R], hd[R];
       col_load4<T, R>(a, b, c, d, es, s, sok, (ch + 1) * CH, n_real, c_pad, ha, hb, hc, hd);
-      inlane_forward_interior<T, R>(ha, hb, hc, hd, KIN);
+      inlane_forward_interior<T, R, true>(ha, hb, hc, hd, KIN);
       col_put_heads<T, R, KIN>(cin, lane, ha, hb, hc, hd);
     }
     const long long i0 = ch * CH + (long long)w * R;
@@ -146,7 +146,7 @@ tdg_col_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
     col_load4<T, R>(a, b, c, d, es, s, sok, i0, n_real, c_pad, ra, rb, rc, rd);
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
     col_put_heads<T, R, KIN>(pg + w * HE, lane, ra, rb, rc, rd);
     __syncthreads();
     Heads<T, R> H;
@@ -206,7 +206,7 @@ tdg_col_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T*
 #pragma unroll
       for (int q = 0; q < Q; ++q) xs[q] = T(0);
     }
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
 #pragma unroll
     for (int q = 0; q < Q; ++q) rd[((q + 1) << KIN) - 1] = xs[q];
     inlane_backward<T, R>(ra, rb, rc, rd, KIN, xprev);
@@ -345,7 +345,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (j == 0 && ch + 1 < C && w == 0) {
       T ha[R], hb[R], hc[R], hd[R];
       col_load4<T, R>(a, b, c, d, es, s, sok, (ch + 1) * CH, n_real, c_pad, ha, hb, hc, hd);
-      inlane_forward_interior<T, R>(ha, hb, hc, hd, KIN);
+      inlane_forward_interior<T, R, true>(ha, hb, hc, hd, KIN);
       col_put_heads<T, R, KIN>(cin, lane, ha, hb, hc, hd);
     }
     const long long i0 = ch * CH + (long long)w * R;
@@ -362,7 +362,7 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     col_fix_ragged<T, R>(sok, i0, n_real, c_pad, ra, rb, rc, rd);
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
     stp.mark(2);
     col_put_heads<T, R, KIN>(pg + w * HE, lane, ra, rb, rc, rd);
     __syncthreads();
@@ -473,7 +473,7 @@ tdg_col_expand_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     col_fix_ragged<T, R>(sok, i0, n_real, c_pad, ra, rb, rc, rd);
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
     stp.mark(2);
 #pragma unroll
     for (int q = 0; q < Q; ++q) rd[((q + 1) << KIN) - 1] = xs[q];

@@ -386,7 +386,7 @@ __device__ __forceinline__ void cta_inlane_forward(T (&ra)[R], T (&rb)[R], T (&r
   const int ls = threadIdx.x;
   const int lane = ls & 31;
   const int warp = ls >> 5;
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, kin);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, kin);
     // Heads: lanes 0..30 take them from lane+1 by shuffle; lane 31 of warp w
     // takes warp w+1's lane 0 through shared memory.
     Heads<T, R> H;

@@ -78,7 +78,7 @@ tdg_large_heads_kernel(const T* __restrict__ a, const T* __restrict__ b, const T
     const long long ch = r - sys * (C - 1) + 1;
     T ra[R], rb[R], rc[R], rd[R];
     large_load4<T, R, true>(a, b, c, d, ss, sys, ch * chunk, n_real, vec, c_pad, ra, rb, rc, rd);
-    inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
     T* h = hbuf + r * (4 * NH);
 #pragma unroll
     for (int l = 1; l <= NH; ++l) {
@@ -101,7 +101,7 @@ __device__ __forceinline__ void large_forward(T (&ra)[R], T (&rb)[R], T (&rc)[R]
                                               const T* hrec, T (*sh)[4]) {
   constexpr int NH = large_heads_elems<R>() / 4;
   const int ls = threadIdx.x, lane = ls & 31, warp = ls >> 5;
-  inlane_forward_interior<T, R>(ra, rb, rc, rd, KIN);
+  inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
   Heads<T, R> H;
   heads_from_next_lane<T, R>(ra, rb, rc, rd, KIN, 32, false, H);
   if (lane == 0 && warp > 0) {
