@@ -375,6 +375,56 @@ def verify(td, a, b, c, d, x, samples, s0):
                    "max|x - x^|/max|x^| (R18); max / sum over ranks"}
 
 
+def scatter_leg(td, args, world, rank, S, n, dt, T, m, reps=5, warmup=2):
+    """scatter (root -> all) + solve + gather (all -> root) of a W * S batch
+    that starts on rank 0; see partition.scatter_solve_gather."""
+    import torch
+    import torch.distributed as dist
+    from paper_conf_ppopp_zhangco10_b200 import inputs
+    from paper_conf_ppopp_zhangco10_b200.partition import reduce_max, scatter_solve_gather
+    root = (inputs.generate(args.family, world * S, n, dt, device="cuda") if rank == 0
+            else (None,) * 4)
+
+    def solve(a, b, c, d):
+        return td.solve_batched(a, b, c, d, algo=args.algo, switch_level=m)
+
+    ph = [0.0, 0.0, 0.0]
+    tot = 0.0
+    for it in range(warmup + reps):
+        ev = [torch.cuda.Event(enable_timing=True) for _ in range(4)]
+        dist.barrier()
+        torch.cuda.synchronize()
+        x_full, _ = scatter_solve_gather(root, (S, n), solve, events=ev)
+        torch.cuda.synchronize()
+        if it >= warmup:
+            for i in range(3):
+                ph[i] += ev[i].elapsed_time(ev[i + 1]) / 1e3
+            tot += ev[0].elapsed_time(ev[3]) / 1e3
+    t = reduce_max(tot / reps)
+    phases = [reduce_max(v / reps) for v in ph]
+    ok = None
+    if rank == 0:
+        # the gathered x is the whole batch's solve: the last shard (solved on
+        # rank W-1) against rank 0 solving the same rows itself, bitwise
+        lo = (world - 1) * S
+        x_ref = td.solve_batched(*[r[lo:] for r in root], algo=args.algo, switch_level=m)
+        ok = bool(torch.equal(x_full[lo:], x_ref))
+    moved = 4 * (world - 1) * S * n * T + (world - 1) * S * n * T
+    del root
+    torch.cuda.empty_cache()
+    return {"value": world * S / t, "unit": UNIT, "systems": world * S,
+            "ms_per_step": 1e3 * t,
+            "phase_ms_max_over_ranks": {"scatter": 1e3 * phases[0], "solve": 1e3 * phases[1],
+                                        "gather": 1e3 * phases[2]},
+            "bytes_over_links_per_step": moved,
+            "link_gbs_root": moved / (phases[0] + phases[2]) / 1e9,
+            "gathered_x_bitwise_equal_to_local_solve": ok,
+            "how": "rank 0 holds all W*S systems; dist.scatter of a, b, c, d (NCCL over "
+                   "NVLink/NVSwitch), solve per rank, dist.gather of x to rank 0; CUDA events "
+                   f"per phase on each rank, {reps} reps after {warmup} warm-up, max over ranks. "
+                   "Context for the paper's with-transfer column (P:L738-746), not the headline."}
+
+
 def pcie_peaks(h, hx, reps=5):
     """Pinned host <-> device copy rates (GB/s, best of `reps`) of one
     buffer the size of d: the ceiling of the host-buffer path."""
@@ -555,6 +605,13 @@ def main():
                 per_algo[key] = {"systems_per_s": sps, "gbs_per_gpu": gbs, "frac_of_peak": gbs / peak,
                                  "family": fam}
         line["per_algo"] = per_algo
+        # --- NVLink "with transfer" context row (NEXT f4; the paper's PCIe
+        # column, as a scatter from one GPU): rank 0 holds the whole
+        # job's batch, scatters equal shards to every rank over NCCL, each rank
+        # solves, x is gathered back to rank 0.  Device time (CUDA events on
+        # each rank's stream), max over ranks.  Only with NCCL (one GPU per rank).
+        if world > 1 and args.dist_backend == "nccl":
+            line["scatter"] = scatter_leg(td, args, world, rank, S, n, dt, T, m)
         # the other BASELINE.json configs (CR+PCR at the tuned m, this rank's GPU):
         # C3 ADI-style 4096 x 4096 (row sweep contiguous, column sweep interleaved),
         # C4 2^20 x 256 on one GPU, C5's largest system n = 8192.

@@ -28,7 +28,9 @@ class TridiagError(RuntimeError):
 
 
 def lib_path() -> str:
-    return _build.LIB
+    # TRIDIAG_LIB_AB: another in-tree build of the same library, for A/B timing
+    # of two builds on one box (tools/ab_bench.py); never set by the product
+    return os.environ.get("TRIDIAG_LIB_AB") or _build.LIB
 
 
 def load(build_if_missing: bool = True) -> ctypes.CDLL:
@@ -37,15 +39,15 @@ def load(build_if_missing: bool = True) -> ctypes.CDLL:
     with _lock:
         if _lib is not None:
             return _lib
-        if build_if_missing:
+        if build_if_missing and not os.environ.get("TRIDIAG_LIB_AB"):
             try:
                 _build.build()
             except (OSError, RuntimeError) as e:  # no nvcc on this machine
                 if not os.path.exists(_build.LIB):
                     raise RuntimeError(f"libtridiag.so is missing and could not be built: {e}")
-        if not os.path.exists(_build.LIB):
-            raise RuntimeError(f"libtridiag.so not found at {_build.LIB}; run __graft_entry__.build()")
-        L = ctypes.CDLL(_build.LIB)
+        if not os.path.exists(lib_path()):
+            raise RuntimeError(f"libtridiag.so not found at {lib_path()}; run __graft_entry__.build()")
+        L = ctypes.CDLL(lib_path())
         P, I64, I = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int
         L.tridiag_solve_batched.argtypes = [P, P, P, P, P, I64, I64, I, I, I, P]
         L.tridiag_solve_batched.restype = I

@@ -95,3 +95,44 @@ def test_gloo_world2_partition_generation_and_reduction():
         assert tmax == 2.0 and tsum == S
         assert total == S and scaling == "strong"
         assert wk == (rank * 5, 5, 10, "weak")
+
+
+def _scatter_worker(rank, world, port, s, n, q):
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle
+        from paper_conf_ppopp_zhangco10_b200.partition import scatter_solve_gather
+        root = inputs.generate("dd", world * s, n, torch.float64) if rank == 0 else (None,) * 4
+
+        def solve(a, b, c, d):
+            return torch.from_numpy(oracle.thomas(*[t.numpy() for t in (a, b, c, d)]))
+
+        x_full, x = scatter_solve_gather(root, (s, n), solve)
+        q.put((rank, None if x_full is None else x_full.numpy(), x.numpy()))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_gloo_world2_scatter_solve_gather():
+    """The NVLink "with transfer" analogue (NEXT f4): the root's batch is
+    scattered in equal shards, solved per rank, gathered back -- the gathered x
+    is the whole-batch solve, and each rank solved exactly its own rows."""
+    world, s, n = 2, 9, 32
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_scatter_worker, args=(r, world, port, s, n, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    out = sorted((q.get(timeout=120) for _ in range(world)), key=lambda o: o[0])
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    import oracle
+    a, b, c, d = inputs.generate("dd", world * s, n, torch.float64)
+    x_whole = oracle.thomas(*[t.numpy() for t in (a, b, c, d)])
+    assert out[1][1] is None
+    assert np.array_equal(out[0][1], x_whole)
+    for rank, _, x in out:
+        assert np.array_equal(x, x_whole[rank * s:(rank + 1) * s])
