@@ -605,13 +605,6 @@ def main():
                 per_algo[key] = {"systems_per_s": sps, "gbs_per_gpu": gbs, "frac_of_peak": gbs / peak,
                                  "family": fam}
         line["per_algo"] = per_algo
-        # --- NVLink "with transfer" context row (NEXT f4; the paper's PCIe
-        # column, P:L738-746, as a scatter from one GPU): rank 0 holds the whole
-        # job's batch, scatters equal shards to every rank over NCCL, each rank
-        # solves, x is gathered back to rank 0.  Device time (CUDA events on
-        # each rank's stream), max over ranks.  Only with NCCL (one GPU per rank).
-        if world > 1 and args.dist_backend == "nccl":
-            line["scatter"] = scatter_leg(td, args, world, rank, S, n, dt, T, m)
         # the other BASELINE.json configs (CR+PCR at the tuned m, this rank's GPU):
         # C3 ADI-style 4096 x 4096 (row sweep contiguous, column sweep interleaved),
         # C4 2^20 x 256 on one GPU, C5's largest system n = 8192.
@@ -665,6 +658,17 @@ def main():
         line["paper_context"] = {"gtx280_cr_pcr_512x512_ms": 0.422,
                                  "gtx280_systems_per_s": 512 / 0.422e-3,
                                  "note": "PAPER.md Fig 15 (P:L1100); context only, not vs_baseline"}
+        # --- NVLink "with transfer" context row (NEXT f4; the paper's PCIe
+        # column, P:L738-746, as a scatter from one GPU): rank 0 holds the whole
+        # job's batch, scatters equal shards to every rank over NCCL, each rank
+        # solves, x is gathered back to rank 0.  Device time (CUDA events on
+        # each rank's stream), max over ranks.  Only with NCCL (one GPU per
+        # rank); last, so that everything above is already in the line.
+        if world > 1 and args.dist_backend == "nccl" and os.environ.get("TRIDIAG_BENCH_SCATTER", "1") != "0":
+            try:
+                line["scatter"] = scatter_leg(td, args, world, rank, S, n, dt, T, m)
+            except Exception as e:  # context row only: keep the line
+                line["scatter"] = {"error": f"{type(e).__name__}: {e}"}
     if world > 1:
         dist.barrier()
         dist.destroy_process_group()
