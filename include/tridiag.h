@@ -191,8 +191,7 @@ size_t tridiag_host_workspace_bytes(int64_t n, int dtype, int64_t chunk_systems)
  * workspace   device buffer owned by the caller, >= tridiag_large_workspace_bytes
  *             bytes (256-byte aligned for the vector path; NULL allowed when
  *             that is 0).  Holds the reduced systems (4 arrays per level, the
- *             deepest one solved in place) and the chunk-boundary head
- *             equations; about 4 S n T / (R - 1) bytes.
+ *             deepest one solved in place); about 4 S n T / (R - 1) bytes.
  * Asynchronous on `stream` like tridiag_solve_batched; x == d allowed.
  */
 int tridiag_solve_batched_large(const void* a, const void* b, const void* c, const void* d,

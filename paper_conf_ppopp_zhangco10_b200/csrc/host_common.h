@@ -116,15 +116,15 @@ cudaError_t dispatch_t(const void* a, const void* b, const void* c, const void* 
                        int64_t n, int64_t S, int k, cudaStream_t st, int dtype, int64_t nr,
                        Layout L);
 
-// Large-n passes (tridiag_large.cuh, inst_large.cu).  which: 0 = heads of
-// every chunk boundary into hbuf, 1 = reduction (a, b, c, d) -> (o0..o3),
-// 2 = expansion writing x to o0 from the survivors' solution x2.  n = padded
+// Large-n passes (tridiag_large.cuh, inst_large.cu).  which: 1 = reduction
+// (a, b, c, d) -> (o0..o3), 2 = expansion writing x to o0 from the
+// survivors' solution x2.  n = padded
 // size of this level, n_real / ss = stored equations / system stride.
 template <typename T>
 int64_t large_chunk();
 template <typename T>
 cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d, T* o0, T* o1,
-                       T* o2, T* o3, const T* x2, T* hbuf, int64_t n, int64_t n_real, int64_t ss,
+                       T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t ss,
                        int64_t S, int kin, bool vec, T c_pad, cudaStream_t st);
 
 // Interleaved-layout (ADI column sweep) passes (tridiag_colpass.cuh,

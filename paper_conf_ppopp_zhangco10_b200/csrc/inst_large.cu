@@ -26,7 +26,7 @@ int64_t large_chunk() { return 32LL * kLargeW * large_R<T>(); }
 
 template <typename T>
 cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d, T* o0, T* o1,
-                       T* o2, T* o3, const T* x2, T* hbuf, int64_t n, int64_t n_real, int64_t ss,
+                       T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t ss,
                        int64_t S, int kin, bool vec, T c_pad, cudaStream_t st) {
   constexpr int R = large_R<T>();
   constexpr int W = kLargeW;
@@ -37,26 +37,18 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
   // KIN is a template parameter (survivor slots are compile-time indices)
   auto pick = [&](auto kin_c) -> cudaError_t {
     constexpr int K = decltype(kin_c)::value;
-    if (which == 0) {
-      if (C < 2) return cudaSuccess;
-      auto kern = tdg::tdg_large_heads_kernel<T, R, K>;
-      const int64_t units = S * (C - 1);
-      const int grid = (int)std::min<int64_t>((units + 127) / 128, 148LL * 16);
-      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(128), 0, st, a, b, c, d, hbuf, n, n_real, ss, S, (int)CH, vec ? 1 :
-          0, c_pad);
-      if (lerr != cudaSuccess) return lerr;
-    } else if (which == 1) {
+    if (which == 1) {
       auto kern = tdg::tdg_large_reduce_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
       long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
-      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, o1, o2, o3, hbuf, n, n_real, ss, S,
+      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, o1, o2, o3, n, n_real, ss, S,
           vec ? 1 : 0, c_pad, stamps);
       if (lerr != cudaSuccess) return lerr;
     } else {
       auto kern = tdg::tdg_large_expand_kernel<T, R, W, K>;
       const int grid = persistent_grid<T>((const void*)kern, 32 * W, S * C);
       long long* stamps = stamp_buffer((int64_t)grid * tdg::kStampSystems * tdg::kStampSlots);
-      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, hbuf, n, n_real, ss, S, vec ? 1
+      const cudaError_t lerr = launch_k(kern, dim3(grid), dim3(32 * W), 0, st, a, b, c, d, o0, x2, n, n_real, ss, S, vec ? 1
           : 0, c_pad, stamps);
       if (lerr != cudaSuccess) return lerr;
     }
@@ -75,11 +67,11 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
 template int64_t large_chunk<float>();
 template int64_t large_chunk<double>();
 template cudaError_t large_pass<float>(int, const float*, const float*, const float*, const float*,
-                                       float*, float*, float*, float*, const float*, float*, int64_t,
+                                       float*, float*, float*, float*, const float*, int64_t,
                                        int64_t, int64_t, int64_t, int, bool, float, cudaStream_t);
 template cudaError_t large_pass<double>(int, const double*, const double*, const double*,
                                         const double*, double*, double*, double*, double*,
-                                        const double*, double*, int64_t, int64_t, int64_t, int64_t,
+                                        const double*, int64_t, int64_t, int64_t, int64_t,
                                         int, bool, double, cudaStream_t);
 
 }  // namespace tdg_host

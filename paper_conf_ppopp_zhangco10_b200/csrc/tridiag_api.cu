@@ -369,12 +369,9 @@ int64_t large_m(int64_t np, int dtype, int algo, int64_t m_req, int64_t bottom_n
 
 size_t large_ws_bytes(const std::vector<LargeLevel>& lv, int64_t S, int dtype) {
   const size_t T = elem_size(dtype);
-  const int64_t CH = large_chunk_n(dtype);
-  const int NH = ilog2_64(large_R(dtype));
   size_t total = 0;
   for (const LargeLevel& L : lv) {
     total += 4 * align256((size_t)S * (size_t)(L.n >> L.kin) * T);
-    total += align256((size_t)S * (size_t)(L.n / CH - 1) * 4 * NH * T);
   }
   return total;
 }
@@ -383,10 +380,8 @@ template <typename T>
 int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr, int64_t S,
                   int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
                   int64_t n_last, char* ws, cudaStream_t st, int64_t ss0) {
-  const int64_t CH = large_chunk_n(dtype);
-  const int NH = ilog2_64(large_R(dtype));
   const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
-  struct Buf { T* a; T* b; T* c; T* d; T* h; };
+  struct Buf { T* a; T* b; T* c; T* d; };
   std::vector<Buf> bufs;
   char* p = ws;
   for (const LargeLevel& L : lv) {
@@ -395,8 +390,6 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     B.a = reinterpret_cast<T*>(p); B.b = reinterpret_cast<T*>(p + arr);
     B.c = reinterpret_cast<T*>(p + 2 * arr); B.d = reinterpret_cast<T*>(p + 3 * arr);
     p += 4 * arr;
-    B.h = reinterpret_cast<T*>(p);
-    p += align256((size_t)S * (size_t)(L.n / CH - 1) * 4 * NH * sizeof(T));
     bufs.push_back(B);
   }
   auto al = [](const void* q) { return (reinterpret_cast<uintptr_t>(q) % 32) == 0; };
@@ -414,13 +407,10 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) &&
                      ((uint64_t)ss * sizeof(T)) % 32 == 0;
     const Buf& B = bufs[j];
-    cudaError_t e = large_pass<T>(0, ia, ib, ic, id, nullptr, nullptr, nullptr, nullptr, nullptr,
-                                  B.h, L.n, n_real, ss, S, L.kin, vec, c_pad, st);
-    if (e == cudaSuccess)
-      e = large_pass<T>(1, ia, ib, ic, id, B.a, B.b, B.c, B.d, nullptr, B.h, L.n, n_real, ss, S,
-                        L.kin, vec, c_pad, st);
+    const cudaError_t e = large_pass<T>(1, ia, ib, ic, id, B.a, B.b, B.c, B.d, nullptr, L.n,
+                                        n_real, ss, S, L.kin, vec, c_pad, st);
     if (e != cudaSuccess) return (int)e;
-    launches += (L.n / CH >= 2 ? 1 : 0) + 1;
+    launches += 1;
   }
   // on-chip solve of the reduced system, in place (x == d)
   const Buf& Z = bufs.back();
@@ -441,8 +431,7 @@ int solve_large_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t 
     const bool vec = n_real == L.n && al(ia) && al(ib) && al(ic) && al(id) && al(ox) &&
                      ((uint64_t)ss * sizeof(T)) % 32 == 0;
     const cudaError_t e = large_pass<T>(2, ia, ib, ic, id, ox, nullptr, nullptr, nullptr,
-                                        bufs[jj].d, bufs[jj].h, L.n, n_real, ss, S, L.kin, vec,
-                                        c_pad, st);
+                                        bufs[jj].d, L.n, n_real, ss, S, L.kin, vec, c_pad, st);
     if (e != cudaSuccess) return (int)e;
     launches += 1;
   }

@@ -15,10 +15,14 @@
 // of W warps, R equations per lane exactly as in the on-chip kernels.  The
 // chunk's last lane needs, at every level, the level-(l-1) state of the next
 // chunk's head equation 2^(l-1) - 1; those depend only on the next chunk's
-// first R equations, so a small pass (tdg_large_heads_kernel) computes them
-// once per chunk boundary into the workspace, and both the reduction and the
-// expansion read them from there.  No unit reads another unit's slice, so the
-// expansion may overwrite d with x in place.
+// first R equations.  Each CTA of the reduction pass walks a contiguous range
+// of units in DESCENDING order, so the heads it needs are the ones its
+// previous unit's first lane produced (carried in shared memory); only the
+// first unit of a CTA computes them from the next chunk's first R equations
+// (round 2: this replaced a separate heads pass per level).  The expansion
+// pass needs no heads at all: the tail chain only changes each lane's tail, a
+// survivor whose x comes from the reduced solve.  No unit reads another unit's
+// output, so the expansion may overwrite d with x in place.
 #pragma once
 
 #include "tridiag_kernels.cuh"  // Stamp
@@ -59,39 +63,6 @@ __device__ __forceinline__ void large_load4(const T* a, const T* b, const T* c, 
 // Heads record per chunk boundary: NH levels x (a, 1/b, c, d).
 template <int R>
 __host__ __device__ constexpr int large_heads_elems() { return 4 * (ilog2c(R) > 0 ? ilog2c(R) : 1); }
-
-// One thread per chunk boundary (sys, ch), ch = 1..C-1: the head equations of
-// chunk ch's first lane after KIN in-lane levels, stored at record
-// sys * (C - 1) + ch - 1 for the last lane of chunk ch - 1.
-template <typename T, int R, int KIN>
-__global__ void __launch_bounds__(128)
-tdg_large_heads_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                       const T* __restrict__ d, T* __restrict__ hbuf, long long n, long long n_real,
-                       long long ss, long long S, int chunk, int vec, T c_pad) {
-  pdl_entry();
-  constexpr int NH = large_heads_elems<R>() / 4;
-  const long long C = n / chunk;
-  const long long total = S * (C - 1);
-  for (long long r = blockIdx.x * (long long)blockDim.x + threadIdx.x; r < total;
-       r += (long long)gridDim.x * blockDim.x) {
-    const long long sys = r / (C - 1);
-    const long long ch = r - sys * (C - 1) + 1;
-    T ra[R], rb[R], rc[R], rd[R];
-    large_load4<T, R, true>(a, b, c, d, ss, sys, ch * chunk, n_real, vec, c_pad, ra, rb, rc, rd);
-    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
-    T* h = hbuf + r * (4 * NH);
-#pragma unroll
-    for (int l = 1; l <= NH; ++l) {
-      if (l <= KIN) {
-        const int t = (1 << (l - 1)) - 1;
-        h[4 * (l - 1) + 0] = ra[t];
-        h[4 * (l - 1) + 1] = rb[t];
-        h[4 * (l - 1) + 2] = rc[t];
-        h[4 * (l - 1) + 3] = rd[t];
-      }
-    }
-  }
-}
 
 // KIN in-lane CR levels of the lane's R equations, completed across lanes,
 // warps (shared memory) and chunks (hbuf); on return the arrays hold the
@@ -135,25 +106,30 @@ __device__ __forceinline__ void large_forward(T (&ra)[R], T (&rb)[R], T (&rc)[R]
 }
 
 // Reduction pass: (a, b, c, d) level j -> survivors (a2, b2, c2, d2) level
-// j + 1, n2 = n >> KIN equations per system, contiguous.
+// j + 1, n2 = n >> KIN equations per system, contiguous.  CTA c walks units
+// [c U / grid, (c + 1) U / grid) from the last to the first (see the header:
+// the next chunk's heads are carried from the previous unit).
 template <typename T, int R, int W, int KIN>
 __global__ void __launch_bounds__(W * 32)
 tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                         const T* __restrict__ d, T* __restrict__ a2, T* __restrict__ b2,
-                        T* __restrict__ c2, T* __restrict__ d2, const T* __restrict__ hbuf,
-                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad,
-                        long long* stamps) {
+                        T* __restrict__ c2, T* __restrict__ d2, long long n, long long n_real,
+                        long long ss, long long S, int vec, T c_pad, long long* stamps) {
   pdl_entry();
   constexpr int P = 32 * W;
   constexpr int NH = large_heads_elems<R>() / 4;
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)P * R;
   __shared__ T sh[W * NH][4];
+  __shared__ T carry[2][4 * NH];   // heads of the chunk walked last (its first lane)
   const long long C = n / CH;
   const long long n2 = n >> KIN;
+  const long long U = S * C;
+  const long long lo = (long long)blockIdx.x * U / gridDim.x;
+  const long long hi = ((long long)blockIdx.x + 1) * U / gridDim.x;
   const int ls = threadIdx.x;
   int j = 0;
-  for (long long u = blockIdx.x; u < S * C; u += gridDim.x, ++j) {
+  for (long long u = hi - 1; u >= lo; --u, ++j) {
     // phase stamps (NEXT f4), warp 0, first kStampSystems units: [0] unit
     // start, [1] loads + KIN forward levels (lanes, warps, chunk heads),
     // [2] survivors stored
@@ -163,13 +139,41 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
     stp.mark(0);
     const long long sys = u / C, ch = u - sys * C;
     const long long i0 = ch * CH + (long long)ls * R;
+    T* cnext = carry[(j + 1) & 1];   // heads of chunk ch + 1
+    if (j == 0 && ch + 1 < C && ls == 0) {
+      // first unit of this CTA: the next chunk's heads from its first R equations
+      T ha[R], hb[R], hc[R], hd[R];
+      large_load4<T, R, true>(a, b, c, d, ss, sys, (ch + 1) * CH, n_real, vec != 0, c_pad, ha, hb, hc, hd);
+      inlane_forward_interior<T, R, true>(ha, hb, hc, hd, KIN);
+#pragma unroll
+      for (int l = 1; l <= NH; ++l) {
+        if (l <= KIN) {
+          const int t = (1 << (l - 1)) - 1;
+          cnext[4 * (l - 1) + 0] = ha[t]; cnext[4 * (l - 1) + 1] = hb[t];
+          cnext[4 * (l - 1) + 2] = hc[t]; cnext[4 * (l - 1) + 3] = hd[t];
+        }
+      }
+    }
     T ra[R], rb[R], rc[R], rd[R];
     large_load4<T, R, true>(a, b, c, d, ss, sys, i0, n_real, vec != 0, c_pad, ra, rb, rc, rd);
     if (i0 == 0) ra[0] = T(0);
     if (i0 + R == n) rc[R - 1] = T(0);
-    const T* hrec = ch + 1 < C ? hbuf + (sys * (C - 1) + ch) * (4 * NH) : nullptr;
-    large_forward<T, R, W, KIN>(ra, rb, rc, rd, hrec, sh);
+    // (the barrier inside large_forward orders cnext's stores before its reads)
+    large_forward<T, R, W, KIN>(ra, rb, rc, rd, ch + 1 < C ? cnext : nullptr, sh);
     stp.mark(1);
+    if (ls == 0) {
+      // this chunk's heads (its first lane's equations 2^(l-1) - 1, unchanged
+      // by the tail chain) for the next unit, chunk ch - 1
+      T* cme = carry[j & 1];
+#pragma unroll
+      for (int l = 1; l <= NH; ++l) {
+        if (l <= KIN) {
+          const int t = (1 << (l - 1)) - 1;
+          cme[4 * (l - 1) + 0] = ra[t]; cme[4 * (l - 1) + 1] = rb[t];
+          cme[4 * (l - 1) + 2] = rc[t]; cme[4 * (l - 1) + 3] = rd[t];
+        }
+      }
+    }
     const long long o = sys * n2 + (i0 >> KIN);
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
@@ -177,7 +181,7 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
       a2[o + q] = ra[t]; b2[o + q] = rb[t]; c2[o + q] = rc[t]; d2[o + q] = rd[t];
     }
     stp.mark(2);
-    __syncthreads();  // sh is reused by the next unit
+    __syncthreads();  // sh / carry are reused by the next unit
   }
 }
 
@@ -186,15 +190,13 @@ tdg_large_reduce_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
 template <typename T, int R, int W, int KIN>
 __global__ void __launch_bounds__(W * 32)
 tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
-                        const T* d, T* x, const T* __restrict__ x2, const T* __restrict__ hbuf,
-                        long long n, long long n_real, long long ss, long long S, int vec, T c_pad,
+                        const T* d, T* x, const T* __restrict__ x2, long long n,
+                        long long n_real, long long ss, long long S, int vec, T c_pad,
                         long long* stamps) {
   pdl_entry();
   constexpr int P = 32 * W;
-  constexpr int NH = large_heads_elems<R>() / 4;
   constexpr int Q = R >> KIN;
   constexpr long long CH = (long long)P * R;
-  __shared__ T sh[W * NH][4];
   const long long C = n / CH;
   const long long n2 = n >> KIN;
   const int ls = threadIdx.x;
@@ -218,8 +220,9 @@ tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
 #pragma unroll
     for (int q = 0; q < Q; ++q) xs[q] = x2[o + q];
     const T xprev = i0 > 0 ? x2[o - 1] : T(0);
-    const T* hrec = ch + 1 < C ? hbuf + (sys * (C - 1) + ch) * (4 * NH) : nullptr;
-    large_forward<T, R, W, KIN>(ra, rb, rc, rd, hrec, sh);
+    // interior levels only: the tail chain (and the heads it needs) changes
+    // only the tails, survivors whose x comes from x2
+    inlane_forward_interior<T, R, true>(ra, rb, rc, rd, KIN);
     stp.mark(1);
 #pragma unroll
     for (int q = 0; q < Q; ++q) rd[((q + 1) << KIN) - 1] = xs[q];
@@ -234,7 +237,6 @@ tdg_large_expand_kernel(const T* __restrict__ a, const T* __restrict__ b, const 
         if (i0 + t < n_real) xb[i0 + t] = rd[t];
     }
     stp.mark(3);
-    __syncthreads();
   }
 }
 

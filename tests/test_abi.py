@@ -168,15 +168,15 @@ def test_large_n_capacity_and_workspace():
     assert td.large_chunk(F32) == 4096 and td.large_chunk(F64) == 2048
     # fits on chip: no workspace
     assert td.large_workspace_bytes(8192, 10, F32, CR) == 0
-    # n = 2^20 fp32: levels 2^20 -> 2^16 -> 2^12; arrays + heads, 256-B aligned
+    # n = 2^20 fp32: levels 2^20 -> 2^16 -> 2^12; the reduced arrays, 256-B aligned
+    # (the chunk heads live in shared memory since round 2)
     S = 3
     exp = 0
     for nl in (1 << 20, 1 << 16):
         exp += 4 * (-(-S * (nl >> 4) * 4 // 256) * 256)
-        exp += -(-S * (nl // 4096 - 1) * 16 * 4 // 256) * 256
     assert td.large_workspace_bytes(1 << 20, S, F32, CR) == exp
     # hybrids stop reducing at m: CR+PCR m = 4096 at n = 16384 is one 2-level pass
-    assert td.large_workspace_bytes(16384, 1, F32, CR_PCR, 4096) == 4 * 4096 * 4 + 256
+    assert td.large_workspace_bytes(16384, 1, F32, CR_PCR, 4096) == 4 * 4096 * 4
     with pytest.raises(ValueError):
         td.large_workspace_bytes(1 << 31, 1, F32, CR)
 
