@@ -47,12 +47,16 @@ def _stale() -> bool:
 def build(force: bool = False, verbose: bool = False) -> str:
     """Compile libtridiag.so if missing or older than its sources: one nvcc per
     translation unit (in parallel), then one link."""
-    if not force and not _stale():
+    if not force and not _stale() and not os.environ.get("TRIDIAG_BUILD_OUT"):
         return LIB
     from concurrent.futures import ThreadPoolExecutor
     import tempfile
     objdir = tempfile.mkdtemp(prefix="tridiag_build_")
     compile_flags = [f for f in NVCC_FLAGS if f != "-shared"]
+    # development A/B builds only (tools/build_ab.sh): extra -D flags and another
+    # output path; the product build sets neither
+    compile_flags += os.environ.get("TRIDIAG_NVCC_DEFINES", "").split()
+    out = os.environ.get("TRIDIAG_BUILD_OUT") or LIB
 
     def compile_one(src):
         obj = os.path.join(objdir, os.path.splitext(src)[0] + ".o")
@@ -69,7 +73,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
         if res.returncode != 0:
             sys.stderr.write(res.stdout + res.stderr)
             raise RuntimeError(f"nvcc failed building {src}")
-    tmp = LIB + f".tmp{os.getpid()}"
+    tmp = out + f".tmp{os.getpid()}"
     link = [nvcc(), "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-Xcompiler", "-fPIC",
             "-o", tmp, *[obj for _, obj, _ in results]]
     res = subprocess.run(link, capture_output=True, text=True)
@@ -80,8 +84,8 @@ def build(force: bool = False, verbose: bool = False) -> str:
         f.write(log_txt)
     if verbose:
         sys.stderr.write(log_txt)
-    os.replace(tmp, LIB)
-    return LIB
+    os.replace(tmp, out)
+    return out
 
 
 if __name__ == "__main__":

@@ -11,7 +11,17 @@ namespace tdg_host {
 namespace {
 template <typename T>
 constexpr int col_R() { return sizeof(T) == 4 ? 16 : 8; }
-constexpr int kColW = 8;
+// Warps per CTA of the TMA reduction / expansion passes (a unit is 32
+// systems x W R rows); the chunk every level must divide is the larger one.
+#ifndef TDG_COL_RED_W
+#define TDG_COL_RED_W 8
+#endif
+#ifndef TDG_COL_EXP_W
+#define TDG_COL_EXP_W 8
+#endif
+constexpr int kColRedW = TDG_COL_RED_W;
+constexpr int kColExpW = TDG_COL_EXP_W;
+constexpr int kColW = kColRedW > kColExpW ? kColRedW : kColExpW;
 }  // namespace
 
 template <typename T>
@@ -55,41 +65,47 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
   constexpr int LR = tdg::ilog2c(R);
   const int64_t CH = col_chunk<T>();
   if (kin < 1 || kin > LR || n % CH != 0) return cudaErrorInvalidValue;
-  const int64_t units = ((S + 31) / 32) * (n / CH);
   int dev = 0;
   cudaGetDevice(&dev);
+  // TMA passes: units of 32 systems x WP R rows (WP = this pass's warps)
+  const int WP = which == 1 ? kColRedW : kColExpW;
+  const int64_t CHP = (int64_t)WP * R;
+  const int64_t units_p = ((S + 31) / 32) * (n / CHP);
   CUtensorMap mA, mB, mC, mD;
-  const bool tma = col_tma_mode() != 0 && make_col_map<T>(&mA, a, S, n_real, es, (int)CH) &&
-                   make_col_map<T>(&mB, b, S, n_real, es, (int)CH) &&
-                   make_col_map<T>(&mC, c, S, n_real, es, (int)CH) &&
-                   make_col_map<T>(&mD, d, S, n_real, es, (int)CH);
+  const bool tma = col_tma_mode() != 0 && make_col_map<T>(&mA, a, S, n_real, es, (int)CHP) &&
+                   make_col_map<T>(&mB, b, S, n_real, es, (int)CHP) &&
+                   make_col_map<T>(&mC, c, S, n_real, es, (int)CHP) &&
+                   make_col_map<T>(&mD, d, S, n_real, es, (int)CHP);
+  const int64_t units = ((S + 31) / 32) * (n / CH);
   auto pick = [&](auto kin_c) -> cudaError_t {
     constexpr int K = decltype(kin_c)::value;
     if (tma && which == 1) {
-      auto kern = tdg::tdg_col_reduce_tma_kernel<T, R, W, K>;
-      const size_t smem = tdg::col_reduce_tma_smem<T, R, W>();
-      const int occ = occupancy(dev, kern, 32 * W, smem);
+      constexpr int WR = kColRedW;
+      auto kern = tdg::tdg_col_reduce_tma_kernel<T, R, WR, K>;
+      const size_t smem = tdg::col_reduce_tma_smem<T, R, WR>();
+      const int occ = occupancy(dev, kern, 32 * WR, smem);
       if (occ <= 0) return cudaErrorInvalidConfiguration;
-      int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units_p, (int64_t)device_sms(dev) * occ));
       // row-aligned pieces when every group gets at least one CTA
-      const int64_t groups = (S + 31) / 32, C = n / CH;
+      const int64_t groups = (S + 31) / 32, C = n / CHP;
       int pieces = 0;
       if (col_order_mode() && groups <= grid) {
         pieces = (int)std::min<int64_t>(C, grid / groups);
         grid = groups * pieces;
       }
       long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
-      const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, a, b, c, d, o0, o1,
+      const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * WR), smem, st, mA, mB, mC, mD, a, b, c, d, o0, o1,
           o2, o3, n, n_real, es, S, es2, ss2, c_pad, tma_pf_mode(), stamps, pieces);
       if (lerr != cudaSuccess) return lerr;
     } else if (tma) {
-      auto kern = tdg::tdg_col_expand_tma_kernel<T, R, W, K>;
-      const size_t smem = tdg::col_stage_bytes<T, R, W>() + 16;
-      const int occ = occupancy(dev, kern, 32 * W, smem);
+      constexpr int WE = kColExpW;
+      auto kern = tdg::tdg_col_expand_tma_kernel<T, R, WE, K>;
+      const size_t smem = tdg::col_stage_bytes<T, R, WE>() + 16;
+      const int occ = occupancy(dev, kern, 32 * WE, smem);
       if (occ <= 0) return cudaErrorInvalidConfiguration;
-      const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units, (int64_t)device_sms(dev) * occ));
+      const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(units_p, (int64_t)device_sms(dev) * occ));
       long long* stamps = stamp_buffer(grid * tdg::kStampSystems * tdg::kStampSlots);
-      const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * W), smem, st, mA, mB, mC, mD, o0, x2, n, n_real, es,
+      const cudaError_t lerr = launch_k(kern, dim3((unsigned)grid), dim3(32 * WE), smem, st, mA, mB, mC, mD, o0, x2, n, n_real, es,
           S, es2, ss2, c_pad, tma_pf_mode() | (col_order_mode() ? 4 : 0), stamps);
       if (lerr != cudaSuccess) return lerr;
     } else if (which == 1) {
