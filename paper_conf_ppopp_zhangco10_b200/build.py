@@ -15,7 +15,7 @@ SOURCES = ["tridiag_api.cu", "inst_f32_pcr.cu", "inst_f32_rd.cu", "inst_f64_pcr.
            "inst_f64_rd.cu", "inst_f32_stone.cu", "inst_f64_stone.cu", "inst_large.cu", "inst_col.cu",
            "inst_paper.cu"]
 DEPS = SOURCES + ["tridiag_device.cuh", "tridiag_kernels.cuh", "tridiag_tma.cuh",
-                  "tridiag_ileave.cuh", "tridiag_large.cuh", "tridiag_colpass.cuh", "tridiag_colcluster.cuh", "tridiag_paper.cuh", "launch.cuh",
+                  "tridiag_ileave.cuh", "tridiag_large.cuh", "tridiag_colpass.cuh", "tridiag_paper.cuh", "launch.cuh",
                   "host_common.h"]
 
 NVCC_FLAGS = [

@@ -127,14 +127,6 @@ cudaError_t large_pass(int which, const T* a, const T* b, const T* c, const T* d
                        T* o2, T* o3, const T* x2, int64_t n, int64_t n_real, int64_t ss,
                        int64_t S, int kin, bool vec, T c_pad, cudaStream_t st);
 
-// Single-pass cluster column sweep (tridiag_colcluster.cuh, inst_col.cu):
-// *used = false and nothing enqueued when the shape / plan has no instance.
-template <typename T>
-cudaError_t col_cluster(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                        int64_t es, int64_t S, int64_t m, cudaStream_t st, bool* used);
-// Single-pass cluster column kernel enabled (TRIDIAG_COL_CLUSTER, default 1).
-int col_cluster_mode();
-
 // Interleaved-layout (ADI column sweep) passes (tridiag_colpass.cuh,
 // inst_col.cu).  which: 1 = reduction (a, b, c, d) -> (o0..o3), 2 = expansion
 // writing x to o0 from x2.  es = element stride of the input (system stride

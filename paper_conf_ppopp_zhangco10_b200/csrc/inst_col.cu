@@ -2,11 +2,8 @@
 // (tridiag_colpass.cuh) for T = float / double; the level plan and the
 // workspace layout live in tridiag_api.cu (solve_col_t).
 #include <cstdlib>
-#include <map>
-#include <mutex>
 
 #include "host_common.h"
-#include "tridiag_colcluster.cuh"
 #include "tridiag_colpass.cuh"
 
 namespace tdg_host {
@@ -140,105 +137,6 @@ cudaError_t col_pass(int which, const T* a, const T* b, const T* c, const T* d, 
       return cudaErrorInvalidValue;
   }
 }
-
-namespace {
-// One cluster launch of the single-pass column kernel for (CL, KB2).
-template <typename T, int CL, int KB2>
-cudaError_t col_cluster_launch(const CUtensorMap& mA, const CUtensorMap& mB, const CUtensorMap& mC,
-                               const CUtensorMap& mD, T* x, int64_t es, int64_t S, int k2,
-                               cudaStream_t st, bool* used) {
-  constexpr int R = col_R<T>();
-  using G = tdg::ColCluster<T, R, CL>;
-  auto kern = tdg::tdg_col_cluster_kernel<T, R, CL, KB2>;
-  const size_t smem = G::template smem_bytes<KB2>();
-  if (smem > 227 * 1024) return cudaSuccess;  // not used
-  static std::mutex mu;
-  static std::map<int, int> max_clusters;     // per device
-  int dev = 0;
-  cudaGetDevice(&dev);
-  cudaLaunchConfig_t cfg = {};
-  cudaLaunchAttribute at[2];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = CL; at[0].val.clusterDim.y = 1; at[0].val.clusterDim.z = 1;
-  at[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-  at[1].val.programmaticStreamSerializationAllowed = 1;
-  cfg.blockDim = dim3(32 * G::W);
-  cfg.dynamicSmemBytes = smem;
-  cfg.stream = st;
-  cfg.attrs = at;
-  int ncl = 0;
-  {
-    std::lock_guard<std::mutex> lk(mu);
-    auto itc = max_clusters.find(dev);
-    if (itc == max_clusters.end()) {
-      cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-      if (CL > 8) cudaFuncSetAttribute(kern, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
-      cfg.gridDim = dim3(CL * 8);
-      cfg.numAttrs = 1;
-      int nc = 0;
-      if (cudaOccupancyMaxActiveClusters(&nc, kern, &cfg) != cudaSuccess) { cudaGetLastError(); nc = 0; }
-      itc = max_clusters.emplace(dev, nc).first;
-    }
-    ncl = itc->second;
-  }
-  if (ncl <= 0) return cudaSuccess;  // not used: the two-pass path runs
-  const int64_t groups = S / 32;
-  const int64_t nc = std::min<int64_t>(groups, ncl);
-  cfg.gridDim = dim3((unsigned)(nc * CL));
-  cfg.numAttrs = pdl_mode() ? 2 : 1;
-  long long* stamps = stamp_buffer(nc * CL * tdg::kStampSystems * tdg::kStampSlots);
-  if (g_kernel_log_len < kMaxKernelLog) g_kernel_log[g_kernel_log_len++] = reinterpret_cast<const void*>(kern);
-  const cudaError_t e = cudaLaunchKernelEx(&cfg, kern, mA, mB, mC, mD, x, (long long)es, (long long)S, k2, stamps);
-  if (e != cudaSuccess) return e;
-  *used = true;
-  return cudaGetLastError();
-}
-}  // namespace
-
-// Single-pass cluster column sweep (tridiag_colcluster.cuh) when the shape
-// fits: interleaved columns, S a multiple of 32, n = CL 16 R with CL in
-// {4, 8, 16}, CR / CR+PCR (PCR inner) with a compiled reduced-solve plan;
-// *used = false (nothing enqueued) otherwise.
-template <typename T>
-cudaError_t col_cluster(const T* a, const T* b, const T* c, const T* d, T* x, int64_t n,
-                        int64_t es, int64_t S, int64_t m, cudaStream_t st, bool* used) {
-  *used = false;
-  constexpr int R = col_R<T>();
-  constexpr int LR = tdg::ilog2c(R);
-  if (S < 32 || S % 32 != 0 || m < 2 || (m & (m - 1)) != 0) return cudaSuccess;
-  const int64_t CH = (int64_t)tdg::kClusterW * R;
-  if (n % CH != 0) return cudaSuccess;
-  const int64_t CL = n / CH;
-  const int64_t n2 = n / R;
-  if (m > n2) return cudaSuccess;
-  int k2 = 0;
-  while ((m << k2) < n2) ++k2;
-  const int kb2 = k2 >= LR ? -1 : k2;
-  CUtensorMap mA, mB, mC, mD;
-  if (!(make_col_map<T>(&mA, a, S, n, es, (int)CH) && make_col_map<T>(&mB, b, S, n, es, (int)CH) &&
-        make_col_map<T>(&mC, c, S, n, es, (int)CH) && make_col_map<T>(&mD, d, S, n, es, (int)CH)))
-    return cudaSuccess;
-  if constexpr (sizeof(T) == 4) {
-    if (CL == 16 && kb2 == 3) return col_cluster_launch<T, 16, 3>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 16 && kb2 == -1) return col_cluster_launch<T, 16, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 8 && kb2 == 2) return col_cluster_launch<T, 8, 2>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 8 && kb2 == -1) return col_cluster_launch<T, 8, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 4 && kb2 == 1) return col_cluster_launch<T, 4, 1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 4 && kb2 == -1) return col_cluster_launch<T, 4, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-  } else {
-    if (CL == 16 && kb2 == -1) return col_cluster_launch<T, 16, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 8 && kb2 == 2) return col_cluster_launch<T, 8, 2>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 8 && kb2 == -1) return col_cluster_launch<T, 8, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 4 && kb2 == 1) return col_cluster_launch<T, 4, 1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-    if (CL == 4 && kb2 == -1) return col_cluster_launch<T, 4, -1>(mA, mB, mC, mD, x, es, S, k2, st, used);
-  }
-  return cudaSuccess;
-}
-
-template cudaError_t col_cluster<float>(const float*, const float*, const float*, const float*, float*,
-                                        int64_t, int64_t, int64_t, int64_t, cudaStream_t, bool*);
-template cudaError_t col_cluster<double>(const double*, const double*, const double*, const double*,
-                                         double*, int64_t, int64_t, int64_t, int64_t, cudaStream_t, bool*);
 
 template int64_t col_chunk<float>();
 template int64_t col_chunk<double>();

@@ -87,21 +87,19 @@ int auto_m(int64_t n, int dtype, int algo) {
 //   TRIDIAG_PHASE_STAMPS per-phase clock stamps (0)
 //   TRIDIAG_PREWAIT_PF   L2 prefetch of the first system before the PDL wait (1)
 //   TRIDIAG_COL_ORDER    chunk-major unit order of the column expansion pass (1)
-//   TRIDIAG_COL_CLUSTER  single-pass cluster column kernel where it applies (1)
 int env_int(const char* name, int dflt) {
   const char* v = getenv(name);
   return (v && *v) ? atoi(v) : dflt;
 }
 
 enum Knob { kWarpR, kPrefetch, kCtaDbuf, kRagTma, kTmaPf, kSmallCta, kPdl, kTma, kBlockedMinb,
-            kColTma, kPhaseStamps, kPrewaitPf, kColOrder, kColCluster, kNumKnobs };
+            kColTma, kPhaseStamps, kPrewaitPf, kColOrder, kNumKnobs };
 struct KnobDef { const char* name; int dflt; };
 constexpr KnobDef kKnobDefs[kNumKnobs] = {
     {"TRIDIAG_WARP_R", 0},    {"TRIDIAG_PREFETCH", 2},  {"TRIDIAG_CTA_DBUF", 1},
     {"TRIDIAG_RAG_TMA", 1},   {"TRIDIAG_TMA_PF", 0},    {"TRIDIAG_SMALL_CTA", 1},
     {"TRIDIAG_PDL", 1},       {"TRIDIAG_TMA", 1},       {"TRIDIAG_BLOCKED_MINB", 2},
-    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}, {"TRIDIAG_PREWAIT_PF", 1}, {"TRIDIAG_COL_ORDER", 1},
-    {"TRIDIAG_COL_CLUSTER", 1}};
+    {"TRIDIAG_COL_TMA", 1},   {"TRIDIAG_PHASE_STAMPS", 0}, {"TRIDIAG_PREWAIT_PF", 1}, {"TRIDIAG_COL_ORDER", 1}};
 std::atomic<int> g_knobs[kNumKnobs];
 std::once_flag g_knobs_once;
 std::mutex g_knobs_mu;
@@ -132,7 +130,6 @@ int blocked_minb() { return knob(kBlockedMinb); }
 int col_tma_mode() { return knob(kColTma); }
 int prewait_pf_mode() { return knob(kPrewaitPf); }
 int col_order_mode() { return knob(kColOrder); }
-int col_cluster_mode() { return knob(kColCluster); }
 
 // Phase stamps (diagnostic, NEXT f4): one device buffer per launch slot of a
 // call (slot = the launch's index within the call, as in the kernel log),
@@ -525,17 +522,6 @@ int solve_col_t(const T* a, const T* b, const T* c, const T* d, T* x, int64_t nr
                 int64_t es, int dtype, int algo, int64_t m, const std::vector<LargeLevel>& lv,
                 int64_t n_last, char* ws, cudaStream_t st) {
   const T c_pad = (algo == TRIDIAG_CR_RD) ? T(1) : T(0);
-  // one pass level, CR or CR+PCR (PCR inner), the real size a power of two:
-  // the single-pass cluster kernel when it has an instance for the shape
-  if (col_cluster_mode() && lv.size() == 1 && nr == lv[0].n && algo != TRIDIAG_CR_RD) {
-    bool used = false;
-    const cudaError_t e = col_cluster<T>(a, b, c, d, x, nr, es, S, m, st, &used);
-    if (e != cudaSuccess) return (int)e;
-    if (used) {
-      g_last_launches = 1;
-      return TRIDIAG_OK;
-    }
-  }
   struct Buf { T* a; T* b; T* c; T* d; };
   std::vector<Buf> bufs;
   char* p = ws;

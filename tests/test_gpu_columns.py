@@ -243,49 +243,3 @@ def test_column_unit_order_is_bitwise_neutral(dtype, monkeypatch):
         td.reload_knobs()
         assert torch.equal(out["1"], out["0"]), (n, S)
         assert torch.equal(out["1"], td.solve_batched(*rows, algo="cr_pcr")), (n, S)
-
-
-CLUSTER_SHAPES = {torch.float32: (1024, 2048, 4096), torch.float64: (1024, 2048)}
-
-
-@pytest.mark.parametrize("dtype", [torch.float32, torch.float64], ids=["f32", "f64"])
-def test_cluster_column_kernel_bitwise(dtype, monkeypatch):
-    """The single-pass cluster column kernel (tridiag_colcluster.cuh: a cluster
-    of CL CTAs keeps 32 systems x all n rows on chip; n = CL 16 R, S a multiple
-    of 32) runs the same CR updates as the two passes and the same warp_solve
-    on the reduced systems: one launch, bitwise the two-pass x
-    (TRIDIAG_COL_CLUSTER=0) and the contiguous solve, for CR+PCR at the tuned
-    m and CR (m = 2), in place x == d too; G1/G2 against fp64 Thomas."""
-    for n in CLUSTER_SHAPES[dtype]:
-        for S, algo in ((32, "cr_pcr"), (96, "cr_pcr"), (64, "cr")):
-            rows = gen("dd", S, n, dtype, seed=7 * n + S)
-            views = as_columns(rows)
-            x1 = cols_solve(views, algo)
-            names = td.last_kernel_names()
-            assert td.last_launch_count() == 1 and "col_cluster" in names[0], (n, S, algo, names)
-            monkeypatch.setenv("TRIDIAG_COL_CLUSTER", "0")
-            td.reload_knobs()
-            x0 = cols_solve(views, algo)
-            assert "col_cluster" not in " ".join(td.last_kernel_names())
-            monkeypatch.delenv("TRIDIAG_COL_CLUSTER")
-            td.reload_knobs()
-            assert torch.equal(x1, x0), (n, S, algo)
-            assert torch.equal(x1.contiguous(), td.solve_batched(*rows, algo=algo)), (n, S, algo)
-            assert float(np.max(err(*rows, x1.contiguous()))) <= TOL[dtype], (n, S, algo)
-            # in place: x == d
-            dd = views[3].clone()
-            y = cols_solve([*views[:3], dd], algo, x=dd)
-            assert y.data_ptr() == dd.data_ptr() and torch.equal(y, x1), (n, S, algo)
-
-
-def test_cluster_column_kernel_falls_back_when_it_does_not_apply():
-    """Shapes without a cluster instance take the two passes: S not a multiple
-    of 32, ragged n, CR+RD, an explicit m whose reduced solve has no instance."""
-    dtype = torch.float32
-    for n, S, algo, m in ((4096, 40, "cr_pcr", 0), (4000, 64, "cr_pcr", 0), (4096, 64, "cr_rd", 0),
-                          (4096, 64, "cr_pcr", 64)):
-        rows = gen("rdw" if algo == "cr_rd" else "dd", S, n, dtype, seed=n + S + m)
-        x = cols_solve(as_columns(rows), algo, m)
-        assert "col_cluster" not in " ".join(td.last_kernel_names()), (n, S, algo, m)
-        if algo != "cr_rd":
-            assert torch.equal(x.contiguous(), td.solve_batched(*rows, algo=algo, switch_level=m)), (n, S, algo, m)
