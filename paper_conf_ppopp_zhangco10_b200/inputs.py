@@ -79,33 +79,44 @@ def uniform(g: torch.Tensor, seed: int, stream: int) -> torch.Tensor:
     return (h >> 8).to(torch.float64) * (1.0 / (1 << 24))
 
 
-def element_index(S: int, n: int, s0: int = 0, device="cpu") -> torch.Tensor:
+def element_index(S: int, n: int, s0: int = 0, device="cpu", i0: int = 0, count=None) -> torch.Tensor:
     s = torch.arange(s0, s0 + S, dtype=torch.int64, device=device)
-    i = torch.arange(n, dtype=torch.int64, device=device)
+    i = torch.arange(i0, i0 + (n - i0 if count is None else count), dtype=torch.int64, device=device)
     return s[:, None] * n + i[None, :]
 
 
 def generate(family: str, S: int, n: int, dtype=torch.float32, seed: int = DEFAULT_SEED,
-             s0: int = 0, device="cpu", E: float = 1.0, poison_corners: bool = False):
+             s0: int = 0, device="cpu", E: float = 1.0, poison_corners: bool = False,
+             i0: int = 0, count=None):
     """Return (a, b, c, d), each an (S, n) contiguous tensor of ``dtype``.
 
     Values are formed in float64 and rounded once to ``dtype``; systems
     [s0, s0+S) of the global batch are produced.  ``poison_corners`` writes
     NaN into a[:, 0] and c[:, n-1], which no solver may read (reading R1).
+    ``i0`` / ``count``: only equations [i0, i0+count) of each n-equation
+    system, (S, count) tensors bitwise equal to those columns of the full
+    systems (a huge system is generated in pieces; families dd, poi, rdw, cv).
     """
     if family not in FAMILIES:
         raise ValueError(f"unknown family {family!r}; one of {FAMILIES}")
     if S < 0 or n < 1:
         raise ValueError("need S >= 0 and n >= 1")
-    g = element_index(S, n, s0, device)
+    cnt = n - i0 if count is None else count
+    if i0 < 0 or cnt < 0 or i0 + cnt > n:
+        raise ValueError("need 0 <= i0 <= i0 + count <= n")
+    if (i0 != 0 or cnt != n) and (family == "km" or poison_corners):
+        raise ValueError("equation ranges are supported for dd / poi / poi1 / rdw / cv without poisoning")
+    g = element_index(S, n, s0, device, i0, cnt)
     f64 = torch.float64
     if family == "dd":
         a = 2.0 * uniform(g, seed, 0) - 1.0
         c = 2.0 * uniform(g, seed, 1) - 1.0
         a_in = a.clone()
         c_in = c.clone()
-        a_in[:, 0] = 0.0
-        c_in[:, n - 1] = 0.0
+        if i0 == 0 and cnt > 0:
+            a_in[:, 0] = 0.0
+        if i0 + cnt == n and cnt > 0:
+            c_in[:, cnt - 1] = 0.0
         sign = torch.where(uniform(g, seed, 3) < 0.5, -1.0, 1.0).to(f64)
         b = sign * (a_in.abs() + c_in.abs() + 1.0 + uniform(g, seed, 2))
         d = 2.0 * uniform(g, seed, 4) - 1.0

@@ -566,6 +566,11 @@ def _residual_rel(a, b, c, d, x):
     ("C4 2^20 x 256 fp32", torch.float32, 1 << 20, 256, "cr_pcr", "dd", 1e-5, 256),
     ("C5 16384 x 8192 fp32", torch.float32, 16384, 8192, "cr_pcr", "dd", 1e-5, 24),
     ("C5 16384 x 8192 fp32 CR+RD (rdw)", torch.float32, 16384, 8192, "cr_rd", "rdw", 5e-3, 24),
+    # the bench's large-n and ragged rows (other_configs), full size
+    ("large n 64 x 2^20 fp32", torch.float32, 64, 1 << 20, "cr_pcr", "dd", 1e-5, 4),
+    ("large n 32 x 2^20 fp64", torch.float64, 32, 1 << 20, "cr_pcr", "dd", 1e-12, 4),
+    ("ragged 67108 x 1000 fp32", torch.float32, 67108, 1000, "cr_pcr", "dd", 1e-5, 64),
+    ("ragged 134217 x 500 fp32", torch.float32, 134217, 500, "cr_pcr", "dd", 1e-5, 64),
 ])
 def test_full_size_other_configs_sampled(name, dtype, S, n, algo, fam, res_tol, samples):
     """The other BASELINE.json configs at their full sizes, in the launch

@@ -1,5 +1,6 @@
 """The shared seeded input generator (no method arithmetic; CPU only)."""
 import numpy as np
+import pytest
 import torch
 
 from paper_conf_ppopp_zhangco10_b200 import inputs
@@ -69,3 +70,25 @@ def test_uniform_has_24_bits_in_unit_interval():
     assert float(u.min()) >= 0.0 and float(u.max()) < 1.0
     assert torch.all(u * (1 << 24) == torch.floor(u * (1 << 24)))
     assert abs(float(u.mean()) - 0.5) < 0.01
+
+
+@pytest.mark.parametrize("family", ["dd", "poi", "poi1", "rdw", "cv"])
+def test_equation_ranges_are_the_columns_of_the_full_systems(family):
+    """generate(..., i0, count) gives exactly columns [i0, i0+count) of the full
+    (S, n) systems (how a 2^30-equation system is generated in pieces)."""
+    S, n = 3, 100
+    full = inputs.generate(family, S, n, torch.float64, s0=7)
+    for cuts in ((0, 100), (0, 1, 100), (0, 37, 64, 99, 100)):
+        parts = [inputs.generate(family, S, n, torch.float64, s0=7, i0=lo, count=hi - lo)
+                 for lo, hi in zip(cuts, cuts[1:])]
+        for k in range(4):
+            assert torch.equal(torch.cat([p[k] for p in parts], dim=1), full[k]), (family, cuts, k)
+
+
+def test_equation_ranges_rejected_where_unsupported():
+    with pytest.raises(ValueError):
+        inputs.generate("km", 2, 10, i0=2, count=3)
+    with pytest.raises(ValueError):
+        inputs.generate("dd", 2, 10, i0=8, count=3)
+    with pytest.raises(ValueError):
+        inputs.generate("dd", 2, 10, i0=1, count=3, poison_corners=True)
