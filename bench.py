@@ -382,8 +382,16 @@ def scatter_leg(td, args, world, rank, S, n, dt, T, m, reps=5, warmup=2):
     import torch.distributed as dist
     from paper_conf_ppopp_zhangco10_b200 import inputs
     from paper_conf_ppopp_zhangco10_b200.partition import reduce_max, scatter_solve_gather
-    root = (inputs.generate(args.family, world * S, n, dt, device="cuda") if rank == 0
-            else (None,) * 4)
+    root = (None,) * 4
+    if rank == 0:
+        # the whole job's batch on rank 0, generated in 2^26-element pieces
+        # (the generator's fp64 temporaries would need ~80 B per element at once)
+        root = tuple(torch.empty((world * S, n), dtype=dt, device="cuda") for _ in range(4))
+        step = max(1, (1 << 26) // n)
+        for s0 in range(0, world * S, step):
+            cnt = min(step, world * S - s0)
+            for dst, src in zip(root, inputs.generate(args.family, cnt, n, dt, s0=s0, device="cuda")):
+                dst[s0:s0 + cnt] = src
 
     def solve(a, b, c, d):
         return td.solve_batched(a, b, c, d, algo=args.algo, switch_level=m)
