@@ -425,7 +425,7 @@ def scatter_leg(td, args, world, rank, S, n, dt, T, m, reps=5, warmup=2):
             "phase_ms_max_over_ranks": {"scatter": 1e3 * phases[0], "solve": 1e3 * phases[1],
                                         "gather": 1e3 * phases[2]},
             "bytes_over_links_per_step": moved,
-            "link_gbs_root": moved / (phases[0] + phases[2]) / 1e9,
+            "link_gbs_root": moved / max(phases[0] + phases[2], 1e-12) / 1e9,
             "gathered_x_bitwise_equal_to_local_solve": ok,
             "how": "rank 0 holds all W*S systems; dist.scatter of a, b, c, d (NCCL over "
                    "NVLink/NVSwitch), solve per rank, dist.gather of x to rank 0; CUDA events "

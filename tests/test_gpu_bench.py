@@ -96,3 +96,37 @@ def test_single_rank_line_certifies_and_names_its_kernel():
     assert chk["oracle_samples_per_rank"] == 256
     assert line["roofline"]["kernel_mangled"].startswith("_Z")
     assert "tdg_warp_kernel" in line["roofline"]["kernel"]
+
+
+_SCATTER_SCRIPT = r"""
+import argparse, json, os, socket, sys
+sys.path.insert(0, os.environ["TDG_ROOT"])
+import torch, torch.distributed as dist
+import bench
+import paper_conf_ppopp_zhangco10_b200 as td
+s = socket.socket(); s.bind(("127.0.0.1", 0)); port = s.getsockname()[1]; s.close()
+torch.cuda.set_device(0)
+dist.init_process_group("nccl", init_method=f"tcp://127.0.0.1:{port}", rank=0, world_size=1,
+                        device_id=torch.device("cuda", 0))
+td.load(build_if_missing=False)
+args = argparse.Namespace(family="dd", algo="cr_pcr")
+out = bench.scatter_leg(td, args, 1, 0, 4096, 512, torch.float32, 4, 32, reps=2, warmup=1)
+dist.destroy_process_group()
+print(json.dumps(out))
+"""
+
+
+def test_scatter_leg_runs_over_nccl_single_rank():
+    """The NVLink with-transfer leg (bench.scatter_leg, NEXT f4) end to end over
+    a real NCCL process group -- of one rank, the only NCCL group a one-GPU box
+    allows (the multi-rank exchange logic is tested with gloo at world size 2
+    in tests/test_dist.py): generation in pieces, dist.scatter / solve /
+    dist.gather, per-phase CUDA events, the bitwise check of the gathered x."""
+    r = subprocess.run([sys.executable, "-c", _SCATTER_SCRIPT], capture_output=True, text=True,
+                       timeout=600, cwd=ROOT, env=dict(os.environ, TDG_ROOT=ROOT))
+    assert r.returncode == 0, r.stderr[-3000:]
+    line = json.loads([ln for ln in r.stdout.splitlines() if ln.startswith("{")][-1])
+    assert line["systems"] == 4096 and line["value"] > 0
+    assert line["gathered_x_bitwise_equal_to_local_solve"] is True
+    assert set(line["phase_ms_max_over_ranks"]) == {"scatter", "solve", "gather"}
+    assert line["bytes_over_links_per_step"] == 0
