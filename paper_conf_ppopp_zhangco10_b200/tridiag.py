@@ -28,9 +28,18 @@ class TridiagError(RuntimeError):
 
 
 def lib_path() -> str:
-    # TRIDIAG_LIB_AB: another in-tree build of the same library, for A/B timing
-    # of two builds on one box (tools/ab_bench.py); never set by the product
-    return os.environ.get("TRIDIAG_LIB_AB") or _build.LIB
+    # TRIDIAG_LIB_AB: another in-tree build of the same library under <repo>/ab/
+    # (tools/build_ab.sh), for A/B timing of two builds on one box
+    # (tools/ab_bench.sh); never set by the product, and nothing outside ab/
+    # is accepted
+    ab = os.environ.get("TRIDIAG_LIB_AB")
+    if not ab:
+        return _build.LIB
+    ab_dir = os.path.realpath(os.path.join(_build.ROOT, "ab"))
+    p = os.path.realpath(ab if os.path.isabs(ab) else os.path.join(_build.ROOT, ab))
+    if os.path.dirname(p) != ab_dir:
+        raise RuntimeError(f"TRIDIAG_LIB_AB must name a build under {ab_dir}")
+    return p
 
 
 def load(build_if_missing: bool = True) -> ctypes.CDLL:
