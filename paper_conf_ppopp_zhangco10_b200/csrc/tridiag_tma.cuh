@@ -220,15 +220,9 @@ tdg_cta_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_constan
     if constexpr (RAG) {
       T* p = x + (size_t)sys * (size_t)ss + (size_t)ls * R;
       if (ls * R + R <= n_real) {
-        // 16-byte aligned (n_real T and R T are multiples of 16 B)
-#pragma unroll
-        for (int q = 0; q < R * (int)sizeof(T) / 16; ++q) {
-          constexpr int E = 16 / (int)sizeof(T);
-          if constexpr (sizeof(T) == 4)
-            *reinterpret_cast<float4*>(p + q * E) = make_float4(rd[q * E], rd[q * E + 1], rd[q * E + 2], rd[q * E + 3]);
-          else
-            *reinterpret_cast<double2*>(p + q * E) = make_double2(rd[q * E], rd[q * E + 1]);
-        }
+        // 16-byte aligned (n_real T and R T are multiples of 16 B): full
+        // 32-byte sectors where the block allows (store_block16)
+        store_block16<T, R>(p, rd);
       } else {
 #pragma unroll
         for (int t = 0; t < R; ++t)
