@@ -242,7 +242,8 @@ __host__ __device__ constexpr size_t col_reduce_tma_smem() {
   // one page of W warps' heads (the unit-start barrier that frees the stage
   // also orders the next unit's head stores after this unit's reads) plus
   // the two carry pages
-  return col_stage_bytes<T, R, W>() + 16 + (size_t)(W + 2) * col_heads_elems<T, R>() * sizeof(T);
+  return col_stage_bytes<T, R, W>() + 16 + (size_t)(W + 2) * col_heads_elems<T, R>() * sizeof(T) +
+         (size_t)4 * W * 32 * sizeof(T);  // survivor tile of the transposed store
 }
 
 template <typename T, int R, int W>
@@ -378,6 +379,29 @@ tdg_col_reduce_tma_kernel(const __grid_constant__ CUtensorMap tmA, const __grid_
     if (w == 0) col_put_heads<T, R, KIN>(carry + (j & 1) * HE, lane, ra, rb, rc, rd);
     inlane_tail_chain<T, R>(ra, rb, rc, rd, KIN, H);
     stp.mark(3);
+    if constexpr (Q == 1 && (W * sizeof(T)) % 32 == 0) {
+      if (es2 == 1) {
+        // the last pass writes its survivors transposed (system s's reduced
+        // row, columns ch W .. ch W + W - 1 from this unit's W warps): through
+        // a [4][W][32] tile so that each lane stores its system's W columns as
+        // whole 32-byte sectors (one warp per array) instead of every warp
+        // storing one 4-byte piece of 32 different sectors
+        T* sv = carry + 2 * HE;
+        sv[(0 * W + w) * 32 + lane] = ra[R - 1]; sv[(1 * W + w) * 32 + lane] = rb[R - 1];
+        sv[(2 * W + w) * 32 + lane] = rc[R - 1]; sv[(3 * W + w) * 32 + lane] = rd[R - 1];
+        __syncthreads();
+        if (w < 4 && sok) {
+          T* outp = (w == 0 ? a2 : w == 1 ? b2 : w == 2 ? c2 : d2) + ((ch * CH) >> KIN) + s * ss2;
+          T v[W];
+#pragma unroll
+          for (int q = 0; q < W; ++q) v[q] = sv[(w * W + q) * 32 + lane];
+#pragma unroll
+          for (int q = 0; q < W * (int)sizeof(T) / 32; ++q) st32B(outp + q * (32 / (int)sizeof(T)), v + q * (32 / (int)sizeof(T)));
+        }
+        stp.mark(4);
+        continue;  // (the next unit's first barrier orders the tile's reuse)
+      }
+    }
     if (sok) {
       const long long o = (i0 >> KIN) * es2 + s * ss2;
 #pragma unroll
