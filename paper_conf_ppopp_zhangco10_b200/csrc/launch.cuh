@@ -15,14 +15,20 @@ cudaError_t launch_ileave_k(const T* a, const T* b, const T* c, const T* d, T* x
                             int64_t S, int k, cudaStream_t st, int64_t n_real, Layout L) {
   const int P = (int)(n / R);
   const int lp = ilog2c(P);
-  const int threads = 1 << tdg::ilv_log_threads(lp);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  // narrow tiles (16-byte row segments: 2^LNS threads at P = 32) when the
+  // default tiles would leave SMs idle (the paper's literal n x n sweeps)
+  constexpr int LNS = 5 + ilog2c(16 / (int)sizeof(T));
+  const bool narrow = lp == 5 && ((S + (512 / 32) - 1) / (512 / 32)) < (int64_t)device_sms(dev) &&
+                      small_cta_mode();
+  const int threads = narrow ? (1 << LNS) : 1 << tdg::ilv_log_threads(lp);
   const int G = threads / P;  // a tile is threads * R elements per array
   const size_t smem = (size_t)5 * tdg::ilv_tile_elems((int)n, G) * sizeof(T);
   if (smem > 227 * 1024) return cudaErrorInvalidValue;
-  int dev = 0;
-  cudaGetDevice(&dev);
   // compile-time geometry for the lane counts the plans use (P = 4 .. 32)
-  auto kern = lp == 5 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 5>
+  auto kern = narrow  ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 5, LNS>
+            : lp == 5 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 5>
             : lp == 4 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 4>
             : lp == 3 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 3>
             : lp == 2 ? tdg::tdg_ileave_kernel<T, R, INNER, KB, 2>

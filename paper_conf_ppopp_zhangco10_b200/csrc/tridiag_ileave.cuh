@@ -46,11 +46,14 @@ __device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wai
 // 512 threads (G = 16 systems, 64-byte fp32 row segments) at P = 32, where
 // 32-byte segments over-fetch from DRAM; 256 threads for smaller P.
 __host__ __device__ constexpr int ilv_log_threads(int lp) { return lp == 5 ? 9 : 8; }
-template <int LP>
+// LNT >= 0: 2^LNT threads instead (the narrow-tile variant for batches with
+// fewer default tiles than SMs: the paper's literal 512 x 512 column sweep has
+// 32 tiles of 16 systems; tiles of 16-byte row segments give 128)
+template <int LP, int LNT = -1>
 struct IlvGeom {
   int lp, lnt;
   __device__ __forceinline__ explicit IlvGeom(int log2P)
-      : lp(LP >= 0 ? LP : log2P), lnt(ilv_log_threads(LP >= 0 ? LP : log2P)) {}
+      : lp(LP >= 0 ? LP : log2P), lnt(LNT >= 0 ? LNT : ilv_log_threads(LP >= 0 ? LP : log2P)) {}
   __device__ __forceinline__ int P() const { return 1 << lp; }
   __device__ __forceinline__ int lg() const { return lnt - lp; }
   __device__ __forceinline__ int G() const { return 1 << (lnt - lp); }
@@ -62,10 +65,10 @@ struct IlvGeom {
 // consecutive systems of a row (whole 32-byte sectors); every offset advances
 // by a constant.  Padding (rows >= n_real, systems >= S, reading R26) and
 // c_{n_real-1} <- c_pad are plain shared stores.
-template <typename T, int R, int LP, bool COPY_D>
+template <typename T, int R, int LP, bool COPY_D, int LNT = -1>
 __device__ __forceinline__ void ilv_issue(const T* a, const T* b, const T* c, const T* d, T* tile,
                                           int TE, long long t0, long long S, int row0, int n_real,
-                                          long long es, const IlvGeom<LP>& Gm, T c_pad) {
+                                          long long es, const IlvGeom<LP, LNT>& Gm, T c_pad) {
   const int G = Gm.G(), P = Gm.P();
   const int g = threadIdx.x & (G - 1);
   const int r0 = threadIdx.x >> Gm.lg();
@@ -135,9 +138,9 @@ __device__ __forceinline__ void ilv_issue(const T* a, const T* b, const T* c, co
 }
 
 // Write the tile's x back: same element mapping, coalesced.
-template <typename T, int R, int LP>
+template <typename T, int R, int LP, int LNT = -1>
 __device__ __forceinline__ void ilv_writeback(T* x, const T* tX, long long t0, long long S, int row0,
-                                              int n_real, long long es, const IlvGeom<LP>& Gm) {
+                                              int n_real, long long es, const IlvGeom<LP, LNT>& Gm) {
   const int G = Gm.G(), P = Gm.P();
   const int g = threadIdx.x & (G - 1);
   const int r0 = threadIdx.x >> Gm.lg();
@@ -168,15 +171,21 @@ __device__ __forceinline__ void ilv_writeback(T* x, const T* tX, long long t0, l
 // same buffer (no registers held while they fly) and overlap the solve; x
 // leaves through the x tile.  5 NT R elements of shared memory: 1 CTA of 16
 // warps (NT = 512) or 2 CTAs of 8 warps per SM.
-template <typename T, int R, int INNER, int KB, int LP>
-__global__ void __launch_bounds__(LP == 5 ? 512 : 256, LP == 5 ? 1 : 2)
+template <int LP, int LNT>
+__host__ __device__ constexpr int ilv_threads() { return LNT >= 0 ? (1 << (LNT >= 0 ? LNT : 0)) : (LP == 5 ? 512 : 256); }
+template <int LP, int LNT>
+__host__ __device__ constexpr int ilv_min_blocks() {
+  return LNT >= 0 ? (65536 / 128) / ilv_threads<LP, LNT>() : (LP == 5 ? 1 : 2);
+}
+template <typename T, int R, int INNER, int KB, int LP, int LNT = -1>
+__global__ void __launch_bounds__(ilv_threads<LP, LNT>(), ilv_min_blocks<LP, LNT>())
 tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __restrict__ c,
                   const T* d, T* x, int n, long long S, int k, int log2P, int n_real, T c_pad,
                   long long es) {
   pdl_entry();
   extern __shared__ __align__(1024) unsigned char smem_raw[];
   T* tile = reinterpret_cast<T*>(smem_raw);
-  const IlvGeom<LP> Gm(log2P);
+  const IlvGeom<LP, LNT> Gm(log2P);
   const int G = Gm.G(), P = Gm.P();
   const int TE = ilv_tile_elems(P * R, G);
   T* tX = tile + 4 * TE;
@@ -189,7 +198,7 @@ tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __r
   const int base = ls * R * G + g + ((ls * R) >> 4);
   const long long tiles = (S + G - 1) / G;
   long long t = blockIdx.x;
-  if (t < tiles) ilv_issue<T, R, LP, true>(a, b, c, d, tile, TE, t * G, S, 0, n_real, es, Gm, c_pad);
+  if (t < tiles) ilv_issue<T, R, LP, true, LNT>(a, b, c, d, tile, TE, t * G, S, 0, n_real, es, Gm, c_pad);
   for (; t < tiles; t += gridDim.x) {
     cp_async_wait_all();
     __syncthreads();  // tile t landed; the x tile's previous write-back is done
@@ -201,14 +210,14 @@ tdg_ileave_kernel(const T* __restrict__ a, const T* __restrict__ b, const T* __r
     }
     __syncthreads();  // every lane holds its rows: the tile buffer is free
     const long long tn = t + gridDim.x;
-    if (tn < tiles) ilv_issue<T, R, LP, true>(a, b, c, d, tile, TE, tn * G, S, 0, n_real, es, Gm, c_pad);
+    if (tn < tiles) ilv_issue<T, R, LP, true, LNT>(a, b, c, d, tile, TE, tn * G, S, 0, n_real, es, Gm, c_pad);
     if (ls == 0) ra[0] = T(0);
     if (ls == P - 1) rc[R - 1] = T(0);
     warp_solve<T, R, INNER, KB>(ra, rb, rc, rd, k, ls, P, Stamp(), pcr_scr);
 #pragma unroll
     for (int q = 0; q < R; ++q) tX[base + q * G] = rd[q];
     __syncthreads();
-    ilv_writeback<T, R, LP>(x, tX, t * G, S, 0, n_real, es, Gm);
+    ilv_writeback<T, R, LP, LNT>(x, tX, t * G, S, 0, n_real, es, Gm);
   }
 }
 
