@@ -453,6 +453,11 @@ __device__ __forceinline__ void cta_inlane_forward(T (&ra)[R], T (&rb)[R], T (&r
 
 }
 
+// Survivor hand-off on a named barrier (producer warps arrive, the solver
+// warp waits) instead of a CTA barrier + warp 0 (A/B: 0 = the round-1 path).
+#ifndef TDG_SURV_NAMED_BARRIER
+#define TDG_SURV_NAMED_BARRIER 1
+#endif
 // Register path (k >= log2 R, m <= 32 lanes or m = survivors): lane-level CR
 // inside every warp, survivors solved by one warp or by the CTA in shared
 // memory, back-substitution.  Returns xprev for the in-lane back-substitution
@@ -528,9 +533,26 @@ __device__ __forceinline__ T cta_register_path(T (&ra)[R], T (&rb)[R], T (&rc)[R
         rd_setup(A, B, C, D, j, msurv, inner + j, msurv);
       }
     }
-    __syncthreads();
+#if TDG_SURV_NAMED_BARRIER
+    // producer / consumer hand-off on named barrier 1: warps 0 .. W-2 arrive
+    // (no wait) once their survivors are stored, the last warp -- under the
+    // oldest-first warp scheduling the last to get there anyway -- waits for
+    // all of them and solves; everyone meets at the barrier that publishes x
+    const int solver = W - 1;
     if (msurv <= 32) {
-      if (warp == 0) {
+      if (warp != solver)
+        asm volatile("bar.arrive 1, %0;" ::"r"(W * 32) : "memory");
+      else
+        asm volatile("bar.sync 1, %0;" ::"r"(W * 32) : "memory");
+    } else {
+      __syncthreads();
+    }
+#else
+    const int solver = 0;
+    __syncthreads();
+#endif
+    if (msurv <= 32) {
+      if (warp == solver) {
         const bool v = lane < msurv;
         const T sA = v ? surv[lane] : T(0), sB = v ? surv[P + lane] : T(1);
         const T sC = v ? surv[2 * P + lane] : T(0), sD = v ? surv[3 * P + lane] : T(0);
